@@ -1,0 +1,312 @@
+"""bench.py -- GStencil-updates/s of the hybrid hexagonal/classical tiled stencil hot path
+on B200 (BASELINE.json metric), with roofline, CPU-oracle baseline and end-to-end numbers.
+
+  python bench.py [--gpus N] [--steps K] [--warmup W] [--config NAME] [--impl reference]
+
+A "step" is one pass of the whole hot path: stencil_run of T time steps over the config's
+synthetic grid (plan built once).  Default config = configs[1] of BASELINE.json: heat /
+laplacian 2D 5-point fp32, 8192^2, T = 512.  N > 1 (torchrun): weak-scaled slab
+decomposition (8192*N x 8192) with halo exchange over torch.distributed/NCCL per time
+block (paper_conf_cgo_grosserchsv14_b200/dist.py).  `--impl reference` times the CPU
+oracle (this tier's reference arm) on the host cores.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import subprocess
+import sys
+import threading
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+CONFIGS = {
+    # name: (kind, extents, T, BASELINE config string)
+    "heat2d5": ("star2d5", (8192, 8192), 512, "heat-2D / laplacian-2D 5-point fp32, 8192x8192, T=512"),
+    "heat2d9": ("box2d9", (8192, 8192), 512, "heat-2D 9-point fp32, 8192x8192, T=512"),
+    "jacobi2d": ("jacobi2d5", (256, 256), 32, "jacobi-2D 5-point fp32, 256x256, T=32"),
+    "fdtd2d": ("fdtd2d", (8192, 8192), 500, "fdtd-2D fp32, 8192x8192, T=500"),
+    "heat3d": ("star3d7", (512, 512, 512), 128, "heat-3D 7-point fp32, 512^3, T=128"),
+    "gradient3d": ("gradient3d", (512, 512, 512), 128, "gradient-3D fp32, 512^3, T=128"),
+}
+METRIC = "GStencil-updates/s (fp32) at 1/2/4/8 B200 and % of time-tiled HBM roofline"
+
+
+def load_peaks():
+    p = os.path.join(ROOT, "MEASURED_PEAKS.json")
+    if os.path.exists(p):
+        d = json.load(open(p))
+        return float(d.get("hbm_gbs", 6650.0)), "measured (MEASURED_PEAKS.json hbm_gbs)"
+    return 6650.0, "fallback (B200_PROFILING.md 6.65 TB/s)"
+
+
+class ClockSampler:
+    """nvidia-smi clocks / throttle reasons sampled every 200 ms during the timed region."""
+
+    FIELDS = ("index,clocks.sm,clocks.max.sm,power.draw,clocks_event_reasons.active,"
+              "clocks_event_reasons.hw_slowdown,clocks_event_reasons.hw_thermal_slowdown,"
+              "clocks_event_reasons.sw_thermal_slowdown,clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, index: int):
+        self.index = index
+        self.proc = None
+        self.lines = []
+        self.t = None
+
+    def __enter__(self):
+        try:
+            self.proc = subprocess.Popen(
+                ["nvidia-smi", f"--id={self.index}", f"--query-gpu={self.FIELDS}",
+                 "--format=csv,noheader,nounits", "-lms", "200"],
+                stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
+            self.t = threading.Thread(target=self._read, daemon=True)
+            self.t.start()
+        except (OSError, FileNotFoundError):
+            self.proc = None
+        return self
+
+    def _read(self):
+        for line in self.proc.stdout:
+            self.lines.append(line.strip())
+
+    def __exit__(self, *a):
+        if self.proc is not None:
+            self.proc.terminate()
+            try:
+                self.proc.wait(timeout=5)
+            except subprocess.TimeoutExpired:
+                self.proc.kill()
+
+    def summary(self):
+        sm, mx, reasons = [], None, set()
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        for line in self.lines:
+            f = [x.strip() for x in line.split(",")]
+            if len(f) < 9:
+                continue
+            try:
+                sm.append(float(f[1]))
+                mx = float(f[2])
+            except ValueError:
+                continue
+            for n, v in zip(names, f[5:9]):
+                if v.lower().startswith("active"):
+                    reasons.add(n)
+        if not sm:
+            return {"sm_mhz": None, "sm_max_mhz": mx, "reasons": [], "samples": 0}
+        return {"sm_mhz": float(np.median(sm)), "sm_max_mhz": mx, "reasons": sorted(reasons),
+                "samples": len(sm)}
+
+
+def bytes_per_update_tiled(info, word):
+    """Algorithmic HBM bytes per update of the hybrid schedule: word*(In+Out)/points of the
+    plan's full hexagon per classical column (DESIGN.md roofline)."""
+    return word * (info["tile_in"] + info["tile_out"]) / info["tile_points"]
+
+
+def cpu_baseline(kind, ext, target_s=12.0):
+    """The oracle as it stands on the host cores, on a bounded sample of the workload
+    (same grid, fewer time steps), scaled to GStencil-updates/s."""
+    import oracle
+    import stencil_inputs
+
+    nthreads = oracle.max_threads()
+    if kind == "fdtd2d":
+        f = stencil_inputs.fields(ext, seed=0, n=3)
+        t0 = time.perf_counter()
+        oracle.fdtd(*f, 2, nthreads=nthreads)
+        dt = (time.perf_counter() - t0) / 2
+        steps = max(2, int(target_s / max(dt, 1e-6)))
+        t0 = time.perf_counter()
+        oracle.fdtd(*f, steps, nthreads=nthreads)
+        el = time.perf_counter() - t0
+        upd = ext[0] * ext[1] * steps
+    else:
+        g = stencil_inputs.uniform(ext, seed=0)
+        t0 = time.perf_counter()
+        oracle.run(kind, g, 2, nthreads=nthreads)
+        dt = (time.perf_counter() - t0) / 2
+        steps = max(2, int(target_s / max(dt, 1e-6)))
+        t0 = time.perf_counter()
+        oracle.run(kind, g, steps, nthreads=nthreads)
+        el = time.perf_counter() - t0
+        upd = int(np.prod([e - 2 for e in ext])) * steps
+    shape = "x".join(map(str, ext))
+    return {"value": upd / el / 1e9, "unit": "GStencil-updates/s", "cores": nthreads, "kind": "oracle",
+            "sample": f"{kind} {shape}, {steps} of the workload's time steps ({el:.1f} s, "
+                      f"OpenMP static over the outer dim, fp32)"}
+
+
+def make_inputs(kind, ext, seed=0):
+    import stencil_inputs
+
+    if kind == "fdtd2d":
+        return stencil_inputs.fields(ext, seed=seed, n=3)
+    return [stencil_inputs.uniform(ext, seed=seed)]
+
+
+def run_reference(args, cfg):
+    kind, ext, T, cname = CONFIGS[cfg]
+    rank = int(os.environ.get("RANK", "0"))
+    if rank != 0:
+        return
+    import oracle
+
+    nthreads = oracle.max_threads()
+    fields = make_inputs(kind, ext)
+    # bounded sample per step: the workload's grid for a few of its time steps
+    steps_per = 4 if kind != "fdtd2d" else 2
+    times = []
+    for i in range(args.warmup + args.steps):
+        t0 = time.perf_counter()
+        if kind == "fdtd2d":
+            oracle.fdtd(*fields, steps_per, nthreads=nthreads)
+        else:
+            oracle.run(kind, fields[0], steps_per, nthreads=nthreads)
+        if i >= args.warmup:
+            times.append(time.perf_counter() - t0)
+    upd = (ext[0] * ext[1] if kind == "fdtd2d" else int(np.prod([e - 2 for e in ext]))) * steps_per
+    val = upd * len(times) / sum(times) / 1e9
+    line = {"impl": "reference", "metric": METRIC, "value": val, "unit": "GStencil-updates/s",
+            "n_gpus": args.gpus, "steps": args.steps, "warmup": args.warmup,
+            "ms_per_step": 1e3 * sum(times) / len(times), "higher_is_better": True,
+            "scaling": "weak", "vs_baseline": None, "dtype": "f32", "data": "synthetic",
+            "config": {"workload": cname, "kind": kind, "extents": list(ext), "T": T},
+            "cpu_baseline": {"value": val, "unit": "GStencil-updates/s", "cores": nthreads,
+                             "kind": "oracle",
+                             "sample": f"each step = {steps_per} of the workload's {T} time steps on the full grid"},
+            "e2e": {"value": val, "unit": "GStencil-updates/s", "h2d_bytes_per_step": 0,
+                    "d2h_bytes_per_step": 0}}
+    print(json.dumps(line), flush=True)
+
+
+def run_gpu(args, cfg):
+    import torch
+
+    from paper_conf_cgo_grosserchsv14_b200 import Plan, Stencil
+
+    kind, ext, T, cname = CONFIGS[cfg]
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    if world > 1:
+        from paper_conf_cgo_grosserchsv14_b200 import dist
+
+        return dist.bench_main(args, cfg, CONFIGS, METRIC)
+    torch.cuda.set_device(local)
+    dev = torch.device("cuda", local)
+    fields = make_inputs(kind, ext)
+    st = Stencil(kind, ext)
+    plan = Plan(st, T)
+    info = plan.info
+    host = [torch.from_numpy(f).pin_memory() for f in fields]
+    xin = [h.to(dev) for h in host]
+    xout = [torch.empty_like(x) for x in xin]
+    one = len(xin) == 1
+    stream = torch.cuda.current_stream(dev)
+
+    def step():
+        plan.run(xin[0] if one else xin, xout[0] if one else xout)
+
+    for _ in range(max(3, args.warmup)):
+        step()
+    torch.cuda.synchronize()
+    # ---- device-timed whole-path steps (inputs resident in HBM; 2 x 256 MiB buffers > L2)
+    start, end = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    with ClockSampler(local) as clocks:
+        torch.cuda.synchronize()
+        start.record(stream)
+        for _ in range(args.steps):
+            step()
+        end.record(stream)
+        torch.cuda.synchronize()
+    ms = start.elapsed_time(end) / args.steps
+    updates = info["updates"]
+    value = updates / (ms * 1e-3) / 1e9
+    # ---- per-launch kernel time of the dominant (phase) kernel, live, same stream
+    plan.profile(args.steps)
+    for _ in range(args.steps):
+        step()
+    prof = plan.profile_read()
+    plan.profile(0)
+    word = 4
+    bpu = bytes_per_update_tiled(info, word)
+    n_launch_per_step = info["n_launches"]
+    avg_launch_ms = prof["kernel_ms"] / prof["launches"]
+    # algorithmic bytes of one average launch = updates per launch x bytes/update
+    alg_bytes_per_launch = updates / n_launch_per_step * bpu
+    achieved_gbs = alg_bytes_per_launch / (avg_launch_ms * 1e-3) / 1e9
+    peak, peak_src = load_peaks()
+    # ---- end to end through the public API: pinned H2D of the inputs, run, D2H of result
+    res_host = [torch.empty_like(h).pin_memory() for h in host]
+    torch.cuda.synchronize()
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    e0.record(stream)
+    for _ in range(args.steps):
+        for h, x in zip(host, xin):
+            x.copy_(h, non_blocking=True)
+        step()
+        for r, x in zip(res_host, xout):
+            r.copy_(x, non_blocking=True)
+    e1.record(stream)
+    torch.cuda.synchronize()
+    e2e_ms = e0.elapsed_time(e1) / args.steps
+    nbytes = sum(h.numel() * h.element_size() for h in host)
+    # ---- naive (non-time-tiled) comparator on the same device, for the >= 2x target
+    naive = Plan(st, T, executor="naive")
+    naive.run(xin[0] if one else xin, xout[0] if one else xout)
+    torch.cuda.synchronize()
+    n0, n1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    n0.record(stream)
+    naive.run(xin[0] if one else xin, xout[0] if one else xout)
+    n1.record(stream)
+    torch.cuda.synchronize()
+    naive_gups = updates / (n0.elapsed_time(n1) * 1e-3) / 1e9
+    cpu = None if args.no_cpu else cpu_baseline(kind, ext)
+    tiled_roof = peak * 1e9 / bpu / 1e9  # GUp/s if HBM-bound at the tiled bytes/update
+    line = {
+        "metric": METRIC, "value": value, "unit": "GStencil-updates/s", "n_gpus": 1,
+        "steps": args.steps, "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True,
+        "scaling": "weak", "vs_baseline": None, "dtype": "f32", "data": "synthetic",
+        "config": {"workload": cname, "kind": kind, "extents": list(ext), "T": T,
+                   "tile": {"h": info["h"], "w0": info["w0"], "w1": info["w"][0]},
+                   "l2": "inputs larger than L2 (2 x 256 MiB ping-pong buffers > 126 MB)"},
+        "roofline": {"bound": "hbm", "achieved": achieved_gbs, "peak": peak, "unit": "GB/s",
+                     "frac": achieved_gbs / peak, "traffic": None, "peak_source": peak_src,
+                     "kernel": "fast2d phase kernel" if info["fast_kernel"] else "hybrid phase kernel",
+                     "bytes_per_update": bpu, "avg_launch_ms": avg_launch_ms,
+                     "tiled_hbm_roofline_gups": tiled_roof,
+                     "kernel_share_of_step": prof["kernel_ms"] / args.steps / ms},
+        "cpu_baseline": cpu,
+        "e2e": {"value": updates / (e2e_ms * 1e-3) / 1e9, "unit": "GStencil-updates/s",
+                "h2d_bytes_per_step": nbytes, "d2h_bytes_per_step": nbytes, "ms_per_step": e2e_ms},
+        "gpu_launches": n_launch_per_step * args.steps,
+        "naive_gups": naive_gups, "speedup_vs_naive": value / naive_gups,
+        "clocks": clocks.summary(),
+    }
+    print(json.dumps(line), flush=True)
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=5)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--config", default="heat2d5", choices=sorted(CONFIGS))
+    ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
+    ap.add_argument("--no-cpu", action="store_true", help="skip the CPU oracle baseline")
+    args = ap.parse_args()
+    args.warmup = max(3, args.warmup)
+    if args.impl == "reference":
+        run_reference(args, args.config)
+    else:
+        run_gpu(args, args.config)
+
+
+if __name__ == "__main__":
+    main()

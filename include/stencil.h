@@ -1,0 +1,201 @@
+/*
+ * stencil.h -- C ABI of the B200-native hybrid hexagonal/classical tiled stencil library
+ * (libhexstencil.so).  Implements the data-parallel hot path of Grosser, Cohen,
+ * Holewinski, Sadayappan, Verdoolaege, "Hybrid Hexagonal/Classical Tiling for GPUs",
+ * CGO'14: T time steps of an iterative affine stencil under
+ * the hybrid schedule of Sec. 3.6.
+ *
+ * Conventions for every entry point
+ *   - Returns stencil_status; nothing throws across the boundary.  On failure a
+ *     thread-local message is available from stencil_last_error().
+ *   - Arguments are plain pointers and sizes; no torch or CUDA types appear.  A "device
+ *     pointer" is a CUDA global-memory address on the current device; a "stream" is a
+ *     cudaStream_t passed as void* (NULL = legacy default stream).
+ *   - Grids are dense, row-major, last dimension contiguous ("stride one",
+ *     PAPER.md:636-641), extents listed slow -> fast and INCLUDING the boundary cells.
+ *     Cells within the radius of an edge are Dirichlet: never written.
+ *   - Ownership: the caller owns every device buffer (inputs, outputs and the plan's
+ *     workspace, allocated e.g. with PyTorch).  The library never allocates, frees or
+ *     retains device memory.  Descriptors and plans are library-owned host objects until
+ *     stencil_destroy, immutable after creation; a plan may run on one stream at a time.
+ *   - Errors: argument and feasibility errors are reported synchronously.  Kernel faults
+ *     are asynchronous (sticky CUDA errors) and surface as STENCIL_E_CUDA on a later
+ *     call.  There is no CPU fallback: without a CUDA device stencil_run fails with
+ *     STENCIL_E_CUDA.
+ */
+#ifndef HEXSTENCIL_STENCIL_H
+#define HEXSTENCIL_STENCIL_H
+
+#include <stddef.h>
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+#define STENCIL_ABI_VERSION 1
+
+typedef enum {
+  STENCIL_OK = 0,
+  STENCIL_E_INVALID = 1,          /* bad argument, NULL handle, size/T mismatch */
+  STENCIL_E_UNSUPPORTED = 2,      /* valid request outside what the library implements */
+  STENCIL_E_INFEASIBLE_TILE = 3,  /* tile parameters violate eq. (1) or the kernel's limits */
+  STENCIL_E_OOM = 4,              /* host allocation failed / workspace too small */
+  STENCIL_E_CUDA = 5,             /* CUDA runtime error (incl. no device) */
+  STENCIL_E_NCCL = 6              /* reserved for the multi-GPU layer */
+} stencil_status;
+
+typedef enum { STENCIL_F32 = 0, STENCIL_F64 = 1 } stencil_dtype;
+
+/* Stencil classes (Table 3; per-point expressions in DESIGN.md). */
+typedef enum {
+  STENCIL_JACOBI2D5 = 0,   /* Fig. 1: k*((((c+s)+n)+e)+w), k = coef[0] (0.2)              */
+  STENCIL_STAR2D5 = 1,     /* laplacian/heat 5-pt: c0*c + c1*(((n+s)+w)+e)  (0.5, 0.125)  */
+  STENCIL_BOX2D9 = 2,      /* heat 2D 9-pt: k * row-major sum of the 3x3 box (1/9)        */
+  STENCIL_FDTD2D = 3,      /* three in-place statements ey, ex, hz (0.5, 0.7); 3 fields   */
+  STENCIL_STAR3D7 = 4,     /* laplacian/heat 3D 7-pt: c0*c + c1*(((((n+s)+w)+e)+u)+d)     */
+  STENCIL_GRADIENT3D = 5,  /* c + 1/sqrt(eps + sum_6 (c-nb)^2)   (eps = 1e-2)             */
+  STENCIL_BOX3D27 = 6,     /* heat 3D 27-pt: k * lexicographic sum of the 3x3x3 box (1/27)*/
+  STENCIL_GRADIENT2D = 7   /* c + 1/sqrt(eps + sum_4 (c-nb)^2)   (eps = 1e-2)             */
+} stencil_kind;
+
+typedef struct stencil_desc_s *stencil_desc_t;
+typedef struct stencil_plan_s *stencil_plan_t;
+
+/* Tile parameters of the hybrid schedule (Sec. 3.6: "parameterized with the values
+ * h, w0, ..., wn").  A hexagonal tile spans 2h+2 (canonical) time
+ * levels; w0 is the minimal hexagon width and must satisfy eq. (1);
+ * w[i] is the classical tile width of the (i+1)-th non-hexagonal dimension.  All-zero
+ * h, w0, w = choose defaults.  hex_dim selects the hexagonally tiled spatial dimension
+ * (Sec. 3.6; must not be the innermost one). */
+typedef struct {
+  int32_t h;
+  int32_t w0;
+  int32_t w[3];
+  int32_t hex_dim;
+  int32_t flags; /* STENCIL_EXEC_* */
+} stencil_tile_t;
+
+enum {
+  STENCIL_EXEC_AUTO = 0,    /* fastest implemented hybrid-tiled kernel for the class      */
+  STENCIL_EXEC_GENERIC = 1, /* generic hybrid kernel straight from global memory
+                               (Table 4 configuration (a))                 */
+  STENCIL_EXEC_NAIVE = 2    /* non-time-tiled comparator: one launch per time step       */
+};
+
+/* Create a stencil descriptor.
+ *   dims        2 or 3 (must match the class)
+ *   extents     dims values, slow -> fast, each >= 3 (boundary included)
+ *   kind        stencil class
+ *   radius      1 (every implemented class has radius 1)
+ *   offsets     optional (may be NULL): n_offsets*dims int32 offsets; if given they must
+ *               equal the class's access set (validated, order free)
+ *   coefficients optional (NULL = class defaults): n_coefficients doubles, rounded once
+ *               to the working precision (see stencil_kind for the count and meaning)
+ *   dtype       STENCIL_F32 or STENCIL_F64 (the arithmetic precision)
+ * Host only; does not touch the GPU. */
+stencil_status stencil_desc_create(stencil_desc_t *out, int dims, const int64_t *extents,
+                                   stencil_kind kind, int radius, const int32_t *offsets,
+                                   int n_offsets, const double *coefficients,
+                                   int n_coefficients, stencil_dtype dtype);
+
+/* Dependence analysis (Sec. 3.2-3.3.2): the memory-based dependence
+ * distance vectors of the canonical schedule [k*t+i, s] (RAW, WAR, WAW of the ping-pong
+ * or in-place layout), written as (dtau, ds_0..ds_{dims-1}) int32 rows into `dist`
+ * (capacity `cap` rows); *n receives the count.  Host only. */
+stencil_status stencil_desc_deps(stencil_desc_t desc, int32_t *dist, int cap, int *n);
+
+/* Build an execution plan for T_steps time steps (a2 tile validation, a3 launch table).
+ * tile may be NULL (= defaults).  Host only. */
+stencil_status stencil_plan(stencil_plan_t *out, stencil_desc_t desc, int64_t T_steps,
+                            const stencil_tile_t *tile);
+
+/* Bytes of device workspace the plan needs (the second ping-pong buffer; 0 for the
+ * in-place FDTD class).  The caller allocates it and hands it over with
+ * stencil_plan_set_workspace before stencil_run.  dev_ptr must be 256-B aligned. */
+stencil_status stencil_plan_workspace_size(stencil_plan_t plan, size_t *bytes);
+stencil_status stencil_plan_set_workspace(stencil_plan_t plan, void *dev_ptr, size_t bytes);
+
+/* Run the plan: out = T_steps steps applied to in.
+ *   in, out   arrays of n_fields device pointers (1, or 3 for FDTD in the order
+ *             ex, ey, hz), each the full grid, 16-B aligned.  in may alias out
+ *             (in-place); in is never written otherwise.
+ *   T_steps   must equal the plan's (STENCIL_E_INVALID otherwise); 0 copies in to out.
+ *   stream    cudaStream_t as void*; all work is enqueued on it (asynchronous).
+ * Per launch-table entry (T, p) one phase kernel is launched (host loop over T and the
+ * two phases). */
+stencil_status stencil_run(stencil_plan_t plan, const void *const *in, void *const *out,
+                           int64_t T_steps, void *stream);
+
+/* Destroy a descriptor or plan (tagged handles).  NULL is a no-op.  A plan keeps its own
+ * copy of the descriptor, so destruction order is free. */
+stencil_status stencil_destroy(void *handle);
+
+/* Thread-local message of the last failing call on this thread ("" if none). */
+const char *stencil_last_error(void);
+
+/* ---------------------------------------------------------------------------------
+ * Introspection (host only): used by tests to check the planner against the schedule
+ * oracle and by the bench for the roofline model.
+ * ------------------------------------------------------------------------------- */
+typedef struct {
+  int32_t dims, kind, dtype, n_fields, statements; /* statements k of tau = k*t + i */
+  int32_t hex_dim;
+  int32_t delta0_num, delta0_den, delta1_num, delta1_den; /* cone slopes along hex_dim */
+  int32_t delta_cls[3];  /* classical skews delta1_i for the other dims (slow -> fast) */
+  int32_t h, w0, w[3];   /* effective tile parameters */
+  int32_t H, W;          /* box height 2h+2 and width 2w0+2+floor(d0 h)+floor(d1 h) */
+  int32_t F0, F1;        /* floor(delta0 h), floor(delta1 h) */
+  int32_t executor;      /* STENCIL_EXEC_* actually used */
+  int32_t fast_kernel;   /* 1 if a specialised register-wavefront kernel runs */
+  int64_t n_launches;    /* launch-table entries (kernel launches per run) */
+  int64_t T_steps, tau_levels;
+  int64_t updates;       /* interior points x T_steps (FDTD: point-steps) */
+  int64_t tile_points;   /* instances of one full hexagon per classical column */
+  int64_t tile_in, tile_out; /* In / Out values of one full hexagon per column */
+  size_t workspace_bytes;
+} stencil_plan_info_t;
+
+stencil_status stencil_plan_info(stencil_plan_t plan, stencil_plan_info_t *info);
+
+/* One launch-table entry (a3): the hexagons S0 in [S0_lo, S0_hi] of time tile T and
+ * phase p run in parallel; each covers canonical levels tau = tau0 + a for
+ * a in [a_lo, a_hi]; its local row b is spatial coordinate s0 = S0*W + b - row_off. */
+typedef struct {
+  int64_t T;
+  int32_t phase;
+  int32_t a_lo, a_hi;
+  int64_t tau0;
+  int64_t S0_lo, S0_hi;
+  int64_t row_off;
+} stencil_launch_t;
+
+stencil_status stencil_plan_launches(stencil_plan_t plan, stencil_launch_t *out, int64_t cap,
+                                     int64_t *n);
+
+/* Hexagon row bounds: for a in [0, 2h+1], rows b in [lo[a], hi[a]] (constraints
+ * (6)-(13)).  cap >= 2h+2. */
+stencil_status stencil_plan_hexagon(stencil_plan_t plan, int32_t *lo, int32_t *hi, int32_t cap);
+
+/* Schedule of one instance (canonical time tau, spatial point s[dims]) as the tuple
+ * [T, p, S0, S_1..S_n, t', s'_0, s'_1..s'_n] of Sec. 3.6 (n = dims-1 classical dims in
+ * slow -> fast order excluding hex_dim), written to sched (capacity 2*dims+3). */
+stencil_status stencil_plan_schedule_of(stencil_plan_t plan, int64_t tau, const int64_t *s,
+                                        int64_t *sched);
+
+/* Per-launch device timing (used by bench.py for the roofline's kernel time).
+ * stencil_plan_profile(plan, max_runs) makes the next max_runs stencil_run calls record a
+ * CUDA event pair around every phase-kernel launch on the run's stream (0 disables and
+ * frees the events).  stencil_plan_profile_read synchronises on the recorded events and
+ * returns the summed kernel time (ms), the number of timed launches and the longest
+ * single launch (ms) over the recorded runs, then resets the recorder. */
+stencil_status stencil_plan_profile(stencil_plan_t plan, int max_runs);
+stencil_status stencil_plan_profile_read(stencil_plan_t plan, double *kernel_ms, int64_t *launches,
+                                         double *max_launch_ms);
+
+int stencil_abi_version(void);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* HEXSTENCIL_STENCIL_H */

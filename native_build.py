@@ -1,0 +1,120 @@
+"""Build the native libraries in-tree (no JIT cache, so the .so files travel to the GPU box).
+
+  * paper_conf_cgo_grosserchsv14_b200/lib/libhexstencil.so -- the product: C++ planner +
+    sm_100a CUDA kernels behind include/stencil.h (nvcc -gencode arch=compute_100a,
+    code=sm_100a, --fmad=false for bit-exact parity, -lineinfo).
+  * oracle/liboracle.so -- the CPU oracle (test infrastructure; built here only so the
+    checker exists -- building it is not using it).
+"""
+from __future__ import annotations
+
+import argparse
+import concurrent.futures as cf
+import hashlib
+import os
+import re
+import subprocess
+import sys
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+PKG = os.path.join(ROOT, "paper_conf_cgo_grosserchsv14_b200")
+CSRC = os.path.join(PKG, "csrc")
+KDIR = os.path.join(CSRC, "kernels")
+OBJ = os.path.join(ROOT, "build", "obj")
+LIB = os.path.join(PKG, "lib", "libhexstencil.so")
+NVCC = os.environ.get("NVCC", "/usr/local/cuda/bin/nvcc")
+
+ARCH = ["-gencode", "arch=compute_100a,code=sm_100a"]
+NVFLAGS = ARCH + ["-O3", "-std=c++17", "-lineinfo", "--fmad=false", "-prec-div=true",
+                  "-prec-sqrt=true", "-ftz=false", "-Xcompiler", "-fPIC", "-Xptxas", "-v",
+                  "-I", os.path.join(ROOT, "include")]
+CXXFLAGS = ["-O2", "-std=c++17", "-fPIC", "-ffp-contract=off", "-I", os.path.join(ROOT, "include"),
+            "-I", "/usr/local/cuda/include"]
+
+
+def _variant_ids(header: str, macro: str):
+    txt = open(os.path.join(KDIR, header)).read()
+    body = txt.split(f"#define {macro}(X)", 1)[1].split("#define", 1)[0]
+    return [int(m) for m in re.findall(r"X\((\d+),", body)]
+
+
+def _deps_hash(paths):
+    h = hashlib.sha1()
+    for p in sorted(paths):
+        h.update(open(p, "rb").read())
+    return h.hexdigest()[:16]
+
+
+def _units():
+    """(source, object, extra flags) for every translation unit."""
+    headers = [os.path.join(dp, f) for dp, _, fs in os.walk(CSRC) for f in fs
+               if f.endswith((".h", ".cuh"))] + [os.path.join(ROOT, "include", "stencil.h")]
+    units = []
+    for src in ["desc.cpp", "plan.cpp"]:
+        units.append((os.path.join(CSRC, src), "cxx", []))
+    for src in ["run.cu", "kernels/generic.cu", "kernels/registry.cu"]:
+        units.append((os.path.join(CSRC, src), "nvcc", []))
+    for vid in _variant_ids("fast2d_variants.h", "HEXS_FAST2D_VARIANTS"):
+        units.append((os.path.join(KDIR, "fast2d_inst.cu"), "nvcc", [f"-DHEXS_VARIANT={vid}"]))
+    out = []
+    for src, tool, extra in units:
+        key = _deps_hash([src] + headers) + hashlib.sha1(" ".join(extra).encode()).hexdigest()[:8]
+        name = os.path.relpath(src, CSRC).replace("/", "_") + ("_" + "_".join(e.split("=")[-1] for e in extra) if extra else "")
+        out.append((src, tool, extra, os.path.join(OBJ, f"{name}.{key}.o")))
+    return out
+
+
+def _compile(unit, verbose=False):
+    src, tool, extra, obj = unit
+    if os.path.exists(obj):
+        return obj, ""
+    if tool == "cxx":
+        cmd = ["g++"] + CXXFLAGS + extra + ["-c", src, "-o", obj]
+    else:
+        cmd = [NVCC] + NVFLAGS + extra + ["-c", src, "-o", obj]
+    r = subprocess.run(cmd, capture_output=True, text=True)
+    if r.returncode != 0:
+        raise RuntimeError(f"compile failed: {' '.join(cmd)}\n{r.stdout}\n{r.stderr}")
+    return obj, r.stderr
+
+
+def build_library(jobs: int = 0, verbose: bool = False) -> str:
+    os.makedirs(OBJ, exist_ok=True)
+    os.makedirs(os.path.dirname(LIB), exist_ok=True)
+    units = _units()
+    jobs = jobs or max(1, os.cpu_count() or 1)
+    logs = []
+    with cf.ThreadPoolExecutor(jobs) as ex:
+        for obj, log in ex.map(lambda u: _compile(u, verbose), units):
+            logs.append((obj, log))
+    objs = [u[3] for u in units]
+    stamp = LIB + ".objs"
+    want = "\n".join(objs)
+    if not os.path.exists(LIB) or not os.path.exists(stamp) or open(stamp).read() != want:
+        cmd = [NVCC] + ARCH + ["-shared", "-o", LIB] + objs + ["-lcudart"]
+        subprocess.check_call(cmd)
+        open(stamp, "w").write(want)
+    if verbose:
+        for obj, log in logs:
+            if log:
+                print(f"== {os.path.basename(obj)}\n{log}")
+    return LIB
+
+
+def build_oracle() -> str:
+    sys.path.insert(0, ROOT)
+    import oracle  # noqa: E402  (test infrastructure; building the checker is not using it)
+    return oracle.build()
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("-j", type=int, default=0)
+    ap.add_argument("-v", action="store_true")
+    args = ap.parse_args()
+    print(build_library(args.j, args.v))
+    print(build_oracle())
+
+
+if __name__ == "__main__":
+    main()

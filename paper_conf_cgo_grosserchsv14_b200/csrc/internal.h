@@ -1,0 +1,113 @@
+// internal.h -- library-internal data structures of libhexstencil (host side).
+#pragma once
+#include <cstddef>
+#include <cstdint>
+#include <string>
+#include <vector>
+
+#include "../../include/stencil.h"
+
+namespace hexs {
+
+constexpr uint32_t kDescMagic = 0x48584453u;  // "HXDS"
+constexpr uint32_t kPlanMagic = 0x48585053u;  // "HXPS"
+constexpr int kMaxLevels = 64;                // max 2h+2 supported by the kernels
+
+// A rational number n/d, d > 0, reduced.
+struct Rat {
+  int64_t n = 0, d = 1;
+};
+Rat make_rat(int64_t n, int64_t d);
+bool rat_less(const Rat& a, const Rat& b);
+int64_t floor_div(int64_t a, int64_t b);
+int64_t ceil_div(int64_t a, int64_t b);
+
+// The statement model of Sec. 3.2: an outer time loop around k >= 1
+// perfect nests; statement i writes field `write` at offset 0 and reads `reads`.
+struct Access {
+  int field;
+  int off[3];
+};
+struct Stmt {
+  int write;
+  std::vector<Access> reads;
+  int lo[3];  // domain per dim: [lo, N + hi)
+  int hi[3];
+};
+
+struct Desc {
+  uint32_t magic = kDescMagic;
+  int dims = 0;
+  int64_t ext[3] = {1, 1, 1};
+  int kind = 0;
+  int radius = 1;
+  int dtype = 0;
+  double coef[4] = {0, 0, 0, 0};
+  int ncoef = 0;
+  int nfields = 1;
+  bool pingpong = true;
+  std::vector<Stmt> stmts;
+  size_t elem() const { return dtype == STENCIL_F64 ? 8 : 4; }
+  int64_t points() const { return ext[0] * ext[1] * (dims == 3 ? ext[2] : 1); }
+};
+
+// Distance vectors (dtau, ds...) of the canonical schedule (dependence analysis, a1).
+std::vector<std::vector<int64_t>> dependence_distances(const Desc& d);
+
+struct Launch {
+  int64_t T;
+  int phase;
+  int a_lo, a_hi;
+  int64_t tau0;
+  int64_t S0_lo, S0_hi;
+  int64_t row_off;
+  // classical tile index ranges (generic executor)
+  int64_t Slo[2], Shi[2];
+};
+
+enum Executor { EXEC_GENERIC = 1, EXEC_NAIVE = 2, EXEC_FAST2D = 3, EXEC_FDTD = 4, EXEC_FAST3D = 5 };
+
+struct Plan {
+  uint32_t magic = kPlanMagic;
+  Desc desc;
+  int64_t T_steps = 0, tau_levels = 0;
+  int hd = 0;           // hexagonal dimension
+  int ncls = 0;         // number of classical dims
+  int cls[2] = {0, 0};  // classical dims (slow -> fast)
+  Rat d0, d1;           // cone slopes along hd
+  int dcls[2] = {0, 0}; // integer classical skews delta1_i
+  int h = 0, w0 = 0, w[2] = {1, 1};
+  int H = 0, W = 0, F0 = 0, F1 = 0, c = 0;
+  std::vector<int32_t> lo, hi;  // hexagon rows per level a
+  std::vector<Launch> launches;
+  int executor = EXEC_GENERIC;
+  int variant = 0;  // fast-kernel instantiation id
+  int64_t tile_points = 0, tile_in = 0, tile_out = 0;
+  size_t ws_bytes = 0;
+  void* ws = nullptr;
+  size_t ws_size = 0;
+  // profiling: event pairs around each launch for up to prof_runs runs
+  int prof_runs = 0, prof_used = 0;
+  std::vector<void*> prof_events;  // cudaEvent_t, 2 per launch per run
+  ~Plan();
+};
+
+// Error reporting (thread-local message).
+stencil_status fail(stencil_status s, const std::string& msg);
+void clear_error();
+
+// plan.cpp
+stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* tile, Plan** out);
+bool schedule_of(const Plan& p, int64_t tau, const int64_t* s, int64_t* sched);
+
+// run.cu
+stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* stream);
+
+// Fast-kernel registry (kernels/*.cu): returns variant id >= 0 or -1 if not instantiated.
+int fast2d_variant(int kind, int dtype, int h, int w0);
+int fast2d_chunk_width(int variant);  // classical tile width w1 the kernel streams
+int fdtd_variant(int dtype, int h, int w0);
+int fast3d_variant(int kind, int dtype, int h, int w0);
+int fast3d_tile(int variant, int* wy, int* wx);
+
+}  // namespace hexs

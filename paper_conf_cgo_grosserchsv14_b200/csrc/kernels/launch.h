@@ -1,0 +1,76 @@
+// launch.h -- argument blocks and host-side launchers of the device kernels.
+#pragma once
+#include <cstdint>
+
+#include <cuda_runtime.h>
+
+namespace hexs {
+
+constexpr int kMaxH = 64;
+
+// Generic hybrid kernel (Table 4 configuration (a): hybrid schedule, global memory only).
+struct GenericArgs {
+  void* f[3];      // ping-pong: f[0], f[1]; FDTD: ex, ey, hz (in place)
+  int64_t N[3];    // extents slow -> fast (unused = 1)
+  int64_t st[3];   // element strides
+  int dims, hd, ncls;
+  int cls[2], dcls[2], w[2];
+  int64_t tau0;
+  int a_lo, a_hi;
+  int64_t S0_lo, row_off;
+  int W;
+  int64_t Slo[2], Shi[2];
+  double k0, k1;
+  int32_t lo[kMaxH], hi[kMaxH];
+};
+cudaError_t launch_generic(int kind, int dtype, const GenericArgs& g, int grid, cudaStream_t s);
+
+// Naive one-step kernels (non-time-tiled comparator, K11).
+struct NaiveArgs {
+  const void* src;
+  void* dst;
+  void* f[3];  // FDTD fields
+  int64_t N[3];
+  double k0, k1;
+  int stmt;    // FDTD statement 0 = ey, 1 = ex, 2 = hz
+};
+cudaError_t launch_naive(int kind, int dtype, int dims, const NaiveArgs& a, cudaStream_t s);
+
+// Fast 2D register-wavefront hybrid kernel (jacobi / star5 / box9 / gradient2d).
+struct Fast2DArgs {
+  void* buf[2];
+  int64_t N0, N1;
+  int64_t tau0;
+  int a_lo, a_hi, a_final;  // a_final: level whose outputs are level T_steps (-1: none)
+  int64_t S0_lo, row_off;
+  int W;
+  double k0, k1;
+};
+cudaError_t launch_fast2d(int variant, const Fast2DArgs& a, int grid, cudaStream_t s);
+
+// FDTD-2D fast kernel.
+struct FdtdArgs {
+  void* f[3];  // ex, ey, hz
+  int64_t N0, N1;
+  int64_t tau0;
+  int a_lo, a_hi, a_final;
+  int64_t S0_lo, row_off;
+  int W;
+  double k0, k1;
+};
+cudaError_t launch_fdtd(int variant, const FdtdArgs& a, int grid, cudaStream_t s);
+
+// 3D fast kernel.
+struct Fast3DArgs {
+  void* buf[2];
+  int64_t N0, N1, N2;
+  int64_t tau0;
+  int a_lo, a_hi, a_final;
+  int64_t S0_lo, row_off;
+  int W;
+  double k0, k1;
+  void* scratch;  // carry scratch (if any)
+};
+cudaError_t launch_fast3d(int variant, const Fast3DArgs& a, int grid, cudaStream_t s);
+
+}  // namespace hexs

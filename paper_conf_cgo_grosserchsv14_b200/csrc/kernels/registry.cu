@@ -1,0 +1,48 @@
+// registry.cu -- maps (class, dtype, h, w0) to compiled fast-kernel variants.
+#include "../internal.h"
+#include "../stencil_ops.cuh"
+#include "fast2d_variants.h"
+#include "launch.h"
+
+namespace hexs {
+
+#define HEXS_DECL(id, dc, T_, KIND_, H_, W0_, NW_)                              \
+  cudaError_t launch_fast2d_v##id(const Fast2DArgs& a, int grid, cudaStream_t s); \
+  int fast2d_chunk_v##id();
+HEXS_FAST2D_VARIANTS(HEXS_DECL)
+#undef HEXS_DECL
+
+int fast2d_variant(int kind, int dtype, int h, int w0) {
+#define HEXS_MATCH(id, dc, T_, KIND_, H_, W0_, NW_) \
+  if (kind == KIND_ && dtype == dc && h == H_ && w0 == W0_) return id;
+  HEXS_FAST2D_VARIANTS(HEXS_MATCH)
+#undef HEXS_MATCH
+  return -1;
+}
+
+int fast2d_chunk_width(int variant) {
+  switch (variant) {
+#define HEXS_W(id, dc, T_, KIND_, H_, W0_, NW_) case id: return fast2d_chunk_v##id();
+    HEXS_FAST2D_VARIANTS(HEXS_W)
+#undef HEXS_W
+    default: return 0;
+  }
+}
+
+cudaError_t launch_fast2d(int variant, const Fast2DArgs& a, int grid, cudaStream_t s) {
+  switch (variant) {
+#define HEXS_L(id, dc, T_, KIND_, H_, W0_, NW_) case id: return launch_fast2d_v##id(a, grid, s);
+    HEXS_FAST2D_VARIANTS(HEXS_L)
+#undef HEXS_L
+    default: return cudaErrorInvalidValue;
+  }
+}
+
+// Not yet specialised: FDTD-2D and 3D classes run the generic hybrid kernel.
+int fdtd_variant(int, int, int) { return -1; }
+cudaError_t launch_fdtd(int, const FdtdArgs&, int, cudaStream_t) { return cudaErrorInvalidValue; }
+int fast3d_variant(int, int, int, int) { return -1; }
+int fast3d_tile(int, int* wy, int* wx) { *wy = 0; *wx = 0; return -1; }
+cudaError_t launch_fast3d(int, const Fast3DArgs&, int, cudaStream_t) { return cudaErrorInvalidValue; }
+
+}  // namespace hexs

@@ -1,0 +1,418 @@
+// plan.cpp -- tile-parameter validation (a2) and the hybrid schedule -> launch table (a3).
+//
+// Implements Sec. 3.3-3.6 of the paper for the planner:
+//   cone slopes delta0/delta1 along the hexagonal dimension  (Sec. 3.3.2, Fig. 3)
+//   width bound, eq. (1)
+//   two-phase tile schedule, eqs. (2)-(5); the phase-0 numerator uses floor(delta0 h)
+//   (reading R1 -- the extracted eq. (3) shows floor(delta1 h), which does not
+//   tile the plane when delta0 != delta1)
+//   hexagon constraints (6),(7),(8),(10),(12),(13) in local box coordinates
+//
+//   classical tiling eqs. (14)-(17) with u = the local box row
+//   host loop "repeatedly iterating over two CUDA kernels"
+#include <algorithm>
+#include <climits>
+#include <cmath>
+#include <memory>
+#include <new>
+#include <set>
+#include <string>
+
+#include "internal.h"
+
+namespace hexs {
+
+namespace {
+
+struct Slopes {
+  Rat d0, d1;
+};
+
+// delta0 = max(0, max ds/dt), delta1 = max(0, max -ds/dt) over the distance vectors
+// (Delta s0 <= delta0 Delta t, Delta s0 >= -delta1 Delta t).
+Slopes cone_slopes(const std::vector<std::vector<int64_t>>& dist, int dim) {
+  Slopes s{make_rat(0, 1), make_rat(0, 1)};
+  for (auto& v : dist) {
+    Rat fwd = make_rat(v[1 + dim], v[0]);
+    Rat bwd = make_rat(-v[1 + dim], v[0]);
+    if (rat_less(s.d0, fwd)) s.d0 = fwd;
+    if (rat_less(s.d1, bwd)) s.d1 = bwd;
+  }
+  return s;
+}
+
+int64_t floor_rat_mul(const Rat& r, int64_t h) { return floor_div(r.n * h, r.d); }
+
+// eq. (1): w0 >= max(delta0 + {delta0 h}, delta1 + {delta1 h}) - 1.  Returns the smallest
+// admissible integer w0.
+int64_t w0_bound(const Rat& d0, const Rat& d1, int64_t h) {
+  auto term = [&](const Rat& d) {
+    // d + {d h} - 1 = d + (d h - floor(d h)) - 1, as a rational with denominator d.d
+    int64_t num = d.n + (d.n * h - floor_rat_mul(d, h) * d.d) - d.d;
+    return ceil_div(num, d.d);
+  };
+  return std::max<int64_t>(0, std::max(term(d0), term(d1)));
+}
+
+bool in_hexagon(const Plan& p, int64_t a, int64_t b) {
+  const int64_t n0 = p.d0.n, q0 = p.d0.d, n1 = p.d1.n, q1 = p.d1.d, h = p.h, w0 = p.w0;
+  // (6)  d0 a - b <= (2h+1) d0 - F0
+  if (n0 * a - b * q0 > (2 * h + 1) * n0 - p.F0 * q0) return false;
+  // (7)  a <= 2h+1 ; (13) a >= 0
+  if (a > 2 * h + 1 || a < 0) return false;
+  // (8)  d1 a + b <= (2h+1) d1 + F0 + w0
+  if (n1 * a + b * q1 > (2 * h + 1) * n1 + (p.F0 + w0) * q1) return false;
+  // (10) d1 a + b >= h d1 - (q1-1)/q1
+  if (n1 * a + b * q1 < h * n1 - (q1 - 1)) return false;
+  // (12) d0 a - b >= d0 h - F0 - w0 - F1 - (q0-1)/q0
+  if (n0 * a - b * q0 < h * n0 - (p.F0 + w0 + p.F1) * q0 - (q0 - 1)) return false;
+  return true;
+}
+
+void hexagon_traffic(Plan& p) {
+  std::set<std::pair<int64_t, int64_t>> pts, ins;
+  for (int a = 0; a < p.H; ++a)
+    for (int b = p.lo[a]; b <= p.hi[a]; ++b) pts.insert({a, b});
+  // offsets along the hexagonal dimension read by any statement
+  std::set<int> offs;
+  for (auto& st : p.desc.stmts)
+    for (auto& ac : st.reads) offs.insert(ac.off[p.hd]);
+  int64_t out = 0;
+  for (auto& q : pts) {
+    bool is_out = false;
+    for (int o : offs) {
+      if (!pts.count({q.first - 1, q.second + o})) ins.insert({q.first - 1, q.second + o});
+      if (!pts.count({q.first + 1, q.second - o})) is_out = true;
+    }
+    out += is_out;
+  }
+  p.tile_points = (int64_t)pts.size();
+  p.tile_in = (int64_t)ins.size();
+  p.tile_out = out;
+}
+
+}  // namespace
+
+bool schedule_of(const Plan& p, int64_t tau, const int64_t* s, int64_t* sched) {
+  const int64_t s0 = s[p.hd];
+  for (int ph = 0; ph < 2; ++ph) {
+    int64_t T, n, a;
+    if (ph == 0) {
+      T = floor_div(tau + p.h + 1, p.H);                    // eq. (2)
+      n = s0 + p.F0 + p.w0 + 1 + T * p.c;                    // eq. (3), floor(d0 h)
+      a = tau + p.h + 1 - T * p.H;
+    } else {
+      T = floor_div(tau, p.H);                               // eq. (4)
+      n = s0 + T * p.c;                                      // eq. (5)
+      a = tau - T * p.H;
+    }
+    const int64_t S0 = floor_div(n, p.W), b = n - S0 * p.W;
+    if (b < p.lo[a] || b > p.hi[a]) continue;
+    int k = 0;
+    sched[k++] = T;
+    sched[k++] = ph;
+    sched[k++] = S0;
+    int64_t sp[2] = {0, 0};
+    for (int q = 0; q < p.ncls; ++q) {
+      const int64_t x = s[p.cls[q]] + (int64_t)p.dcls[q] * a;  // eqs. (14), (17)
+      const int64_t Si = floor_div(x, p.w[q]);
+      sched[k++] = Si;
+      sp[q] = x - Si * p.w[q];
+    }
+    sched[k++] = a;
+    sched[k++] = b;
+    for (int q = 0; q < p.ncls; ++q) sched[k++] = sp[q];
+    return true;
+  }
+  return false;
+}
+
+stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* tile, Plan** out) {
+  if (T_steps < 0) return fail(STENCIL_E_INVALID, "stencil_plan: T_steps < 0");
+  Plan* p = new (std::nothrow) Plan();
+  if (!p) return fail(STENCIL_E_OOM, "stencil_plan: out of host memory");
+  std::unique_ptr<Plan> guard(p);
+  p->desc = d;
+  p->T_steps = T_steps;
+  p->tau_levels = T_steps * (int64_t)d.stmts.size();
+  stencil_tile_t t{};
+  if (tile) t = *tile;
+  p->hd = t.hex_dim;
+  if (p->hd < 0 || p->hd >= d.dims - 1)
+    return fail(STENCIL_E_INVALID, "stencil_plan: hex_dim must be a non-innermost dimension (PAPER.md:636-641)");
+  p->ncls = 0;
+  for (int q = 0; q < d.dims; ++q)
+    if (q != p->hd) p->cls[p->ncls++] = q;
+
+  // a1: dependence analysis -> slopes
+  auto dist = dependence_distances(d);
+  Slopes sl = cone_slopes(dist, p->hd);
+  p->d0 = sl.d0;
+  p->d1 = sl.d1;
+  for (int q = 0; q < p->ncls; ++q) {
+    Slopes c = cone_slopes(dist, p->cls[q]);
+    p->dcls[q] = (int)ceil_div(c.d1.n, c.d1.d);  // integer skew >= delta1_i (Sec. 3.4)
+  }
+
+  // a2: tile parameters
+  const int flags = t.flags;
+  bool auto_tile = (t.h == 0 && t.w0 == 0);
+  int h = t.h, w0 = t.w0;
+  const int dtype = d.dtype;
+  if (auto_tile) {
+    if (d.kind == STENCIL_FDTD2D) {
+      h = 5; w0 = 8;  // 12 tau-levels = 4 full steps per tile (h+1 multiple of 3)
+    } else if (d.dims == 2) {
+      h = 3; w0 = 10;
+    } else {
+      h = 2; w0 = 7;  // Table 4 setup
+    }
+  }
+  if (h < 0 || w0 < 0) return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_plan: negative tile parameter");
+  if (2 * h + 2 > kMaxLevels)
+    return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_plan: 2h+2 exceeds the kernels' level limit (64)");
+  const int64_t wb = w0_bound(p->d0, p->d1, h);
+  if (w0 < wb)
+    return fail(STENCIL_E_INFEASIBLE_TILE,
+                "stencil_plan: w0 violates eq. (1): need w0 >= " + std::to_string(wb));
+  p->h = h;
+  p->w0 = w0;
+  p->F0 = (int)floor_rat_mul(p->d0, h);
+  p->F1 = (int)floor_rat_mul(p->d1, h);
+  p->H = 2 * h + 2;
+  p->W = 2 * w0 + 2 + p->F0 + p->F1;
+  p->c = p->F1 - p->F0;
+  p->lo.assign(p->H, 0);
+  p->hi.assign(p->H, -1);
+  for (int a = 0; a < p->H; ++a) {
+    int lo = -1, hi = -2;
+    for (int b = 0; b < p->W; ++b) {
+      if (in_hexagon(*p, a, b)) {
+        if (lo < 0) lo = b;
+        else if (b != hi + 1) return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_plan: non-convex hexagon row");
+        hi = b;
+      }
+    }
+    if (lo < 0) return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_plan: empty hexagon row");
+    p->lo[a] = lo;
+    p->hi[a] = hi;
+  }
+  hexagon_traffic(*p);
+
+  // executor selection
+  int ex = EXEC_GENERIC;
+  p->variant = -1;
+  if (flags == STENCIL_EXEC_NAIVE) {
+    ex = EXEC_NAIVE;
+  } else if (flags == STENCIL_EXEC_AUTO) {
+    if (d.kind == STENCIL_FDTD2D) {
+      p->variant = fdtd_variant(dtype, h, w0);
+      if (p->variant >= 0 && p->hd == 0) ex = EXEC_FDTD;
+    } else if (d.dims == 2) {
+      p->variant = fast2d_variant(d.kind, dtype, h, w0);
+      if (p->variant >= 0 && p->hd == 0 && p->dcls[0] == 1 && p->d0.n == 1 && p->d0.d == 1 &&
+          p->d1.n == 1 && p->d1.d == 1)
+        ex = EXEC_FAST2D;
+    } else {
+      p->variant = fast3d_variant(d.kind, dtype, h, w0);
+      if (p->variant >= 0 && p->hd == 0) ex = EXEC_FAST3D;
+    }
+  } else if (flags != STENCIL_EXEC_GENERIC) {
+    return fail(STENCIL_E_INVALID, "stencil_plan: unknown tile.flags");
+  }
+  p->executor = ex;
+
+  // classical widths
+  for (int q = 0; q < p->ncls; ++q) {
+    int wq = t.w[q];
+    if (ex == EXEC_FAST2D) wq = fast2d_chunk_width(p->variant);
+    else if (ex == EXEC_FAST3D) {
+      int wy = 0, wx = 0;
+      fast3d_tile(p->variant, &wy, &wx);
+      wq = q == 0 ? wy : wx;
+    } else if (wq <= 0) {
+      wq = (q == p->ncls - 1) ? 128 : 4;
+    }
+    if (wq < 1) return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_plan: classical width must be >= 1");
+    p->w[q] = wq;
+  }
+
+  // a3: launch table.  Order (T, 0), (T, 1), T ascending.
+  int64_t dlo[3], dhi[3];
+  for (int q = 0; q < d.dims; ++q) {
+    dlo[q] = INT64_MAX;
+    dhi[q] = INT64_MIN;
+    for (auto& st : d.stmts) {
+      dlo[q] = std::min<int64_t>(dlo[q], st.lo[q]);
+      dhi[q] = std::max<int64_t>(dhi[q], d.ext[q] + st.hi[q] - 1);
+    }
+  }
+  const int64_t L = p->tau_levels;
+  if (ex != EXEC_NAIVE && L > 0) {
+    const int64_t Tmax0 = floor_div(L - 1 + h + 1, p->H), Tmax1 = floor_div(L - 1, p->H);
+    for (int64_t T = 0; T <= std::max(Tmax0, Tmax1); ++T) {
+      for (int ph = 0; ph < 2; ++ph) {
+        if ((ph == 0 && T > Tmax0) || (ph == 1 && T > Tmax1)) continue;
+        Launch ln{};
+        ln.T = T;
+        ln.phase = ph;
+        ln.tau0 = ph == 0 ? T * p->H - (h + 1) : T * p->H;
+        ln.a_lo = (int)std::max<int64_t>(0, -ln.tau0);
+        ln.a_hi = (int)std::min<int64_t>(p->H - 1, L - 1 - ln.tau0);
+        if (ln.a_lo > ln.a_hi) continue;
+        ln.row_off = T * p->c + (ph == 0 ? p->F0 + w0 + 1 : 0);
+        int bmin = INT32_MAX, bmax = INT32_MIN;
+        for (int a = ln.a_lo; a <= ln.a_hi; ++a) {
+          bmin = std::min(bmin, (int)p->lo[a]);
+          bmax = std::max(bmax, (int)p->hi[a]);
+        }
+        const int hd = p->hd;
+        ln.S0_lo = ceil_div(dlo[hd] + ln.row_off - bmax, p->W);
+        ln.S0_hi = floor_div(dhi[hd] + ln.row_off - bmin, p->W);
+        if (ln.S0_lo > ln.S0_hi) continue;
+        for (int q = 0; q < 2; ++q) {
+          ln.Slo[q] = ln.Shi[q] = 0;
+          if (q < p->ncls) {
+            const int dq = p->cls[q];
+            ln.Slo[q] = floor_div(dlo[dq] + (int64_t)p->dcls[q] * ln.a_lo, p->w[q]);
+            ln.Shi[q] = floor_div(dhi[dq] + (int64_t)p->dcls[q] * ln.a_hi, p->w[q]);
+          }
+        }
+        p->launches.push_back(ln);
+      }
+    }
+  }
+
+  // workspace: the second ping-pong buffer, 256-B granular
+  p->ws_bytes = 0;
+  if (d.pingpong && T_steps > 0) p->ws_bytes = ((size_t)d.points() * d.elem() + 255) / 256 * 256;
+  *out = guard.release();
+  return STENCIL_OK;
+}
+
+}  // namespace hexs
+
+using namespace hexs;
+
+static Plan* as_plan(stencil_plan_t h) {
+  Plan* p = reinterpret_cast<Plan*>(h);
+  return (p && p->magic == kPlanMagic) ? p : nullptr;
+}
+
+extern "C" {
+
+stencil_status stencil_plan(stencil_plan_t* out, stencil_desc_t desc, int64_t T_steps,
+                            const stencil_tile_t* tile) {
+  clear_error();
+  if (!out) return fail(STENCIL_E_INVALID, "stencil_plan: out is NULL");
+  *out = nullptr;
+  Desc* d = reinterpret_cast<Desc*>(desc);
+  if (!d || d->magic != kDescMagic) return fail(STENCIL_E_INVALID, "stencil_plan: bad descriptor");
+  Plan* p = nullptr;
+  stencil_status s = build_plan(*d, T_steps, tile, &p);
+  if (s != STENCIL_OK) return s;
+  *out = reinterpret_cast<stencil_plan_t>(p);
+  return STENCIL_OK;
+}
+
+stencil_status stencil_plan_workspace_size(stencil_plan_t plan, size_t* bytes) {
+  clear_error();
+  Plan* p = as_plan(plan);
+  if (!p || !bytes) return fail(STENCIL_E_INVALID, "stencil_plan_workspace_size: bad arguments");
+  *bytes = p->ws_bytes;
+  return STENCIL_OK;
+}
+
+stencil_status stencil_plan_set_workspace(stencil_plan_t plan, void* dev_ptr, size_t bytes) {
+  clear_error();
+  Plan* p = as_plan(plan);
+  if (!p) return fail(STENCIL_E_INVALID, "stencil_plan_set_workspace: bad plan");
+  if (bytes < p->ws_bytes) return fail(STENCIL_E_OOM, "stencil_plan_set_workspace: workspace too small");
+  if (p->ws_bytes && !dev_ptr) return fail(STENCIL_E_INVALID, "stencil_plan_set_workspace: NULL workspace");
+  if (reinterpret_cast<uintptr_t>(dev_ptr) % 256 != 0)
+    return fail(STENCIL_E_INVALID, "stencil_plan_set_workspace: workspace must be 256-B aligned");
+  p->ws = dev_ptr;
+  p->ws_size = bytes;
+  return STENCIL_OK;
+}
+
+stencil_status stencil_plan_info(stencil_plan_t plan, stencil_plan_info_t* info) {
+  clear_error();
+  Plan* p = as_plan(plan);
+  if (!p || !info) return fail(STENCIL_E_INVALID, "stencil_plan_info: bad arguments");
+  stencil_plan_info_t& o = *info;
+  o = stencil_plan_info_t{};
+  const Desc& d = p->desc;
+  o.dims = d.dims;
+  o.kind = d.kind;
+  o.dtype = d.dtype;
+  o.n_fields = d.nfields;
+  o.statements = (int32_t)d.stmts.size();
+  o.hex_dim = p->hd;
+  o.delta0_num = (int32_t)p->d0.n;
+  o.delta0_den = (int32_t)p->d0.d;
+  o.delta1_num = (int32_t)p->d1.n;
+  o.delta1_den = (int32_t)p->d1.d;
+  for (int q = 0; q < 3; ++q) o.delta_cls[q] = q < p->ncls ? p->dcls[q] : 0;
+  o.h = p->h;
+  o.w0 = p->w0;
+  for (int q = 0; q < 3; ++q) o.w[q] = q < p->ncls ? p->w[q] : 0;
+  o.H = p->H;
+  o.W = p->W;
+  o.F0 = p->F0;
+  o.F1 = p->F1;
+  o.executor = p->executor == EXEC_NAIVE ? STENCIL_EXEC_NAIVE
+             : p->executor == EXEC_GENERIC ? STENCIL_EXEC_GENERIC : STENCIL_EXEC_AUTO;
+  o.fast_kernel = (p->executor == EXEC_FAST2D || p->executor == EXEC_FDTD || p->executor == EXEC_FAST3D);
+  o.n_launches = p->executor == EXEC_NAIVE ? p->tau_levels : (int64_t)p->launches.size();
+  o.T_steps = p->T_steps;
+  o.tau_levels = p->tau_levels;
+  int64_t interior = 1;
+  if (d.kind == STENCIL_FDTD2D) interior = d.ext[0] * d.ext[1];
+  else
+    for (int q = 0; q < d.dims; ++q) interior *= (d.ext[q] - 2 * d.radius);
+  o.updates = interior * p->T_steps;
+  o.tile_points = p->tile_points;
+  o.tile_in = p->tile_in;
+  o.tile_out = p->tile_out;
+  o.workspace_bytes = p->ws_bytes;
+  return STENCIL_OK;
+}
+
+stencil_status stencil_plan_launches(stencil_plan_t plan, stencil_launch_t* out, int64_t cap,
+                                     int64_t* n) {
+  clear_error();
+  Plan* p = as_plan(plan);
+  if (!p || !n) return fail(STENCIL_E_INVALID, "stencil_plan_launches: bad arguments");
+  *n = (int64_t)p->launches.size();
+  if (!out) return STENCIL_OK;
+  if (cap < *n) return fail(STENCIL_E_INVALID, "stencil_plan_launches: capacity too small");
+  for (size_t i = 0; i < p->launches.size(); ++i) {
+    const Launch& l = p->launches[i];
+    out[i] = stencil_launch_t{l.T, l.phase, l.a_lo, l.a_hi, l.tau0, l.S0_lo, l.S0_hi, l.row_off};
+  }
+  return STENCIL_OK;
+}
+
+stencil_status stencil_plan_hexagon(stencil_plan_t plan, int32_t* lo, int32_t* hi, int32_t cap) {
+  clear_error();
+  Plan* p = as_plan(plan);
+  if (!p || !lo || !hi || cap < p->H) return fail(STENCIL_E_INVALID, "stencil_plan_hexagon: bad arguments");
+  for (int a = 0; a < p->H; ++a) {
+    lo[a] = p->lo[a];
+    hi[a] = p->hi[a];
+  }
+  return STENCIL_OK;
+}
+
+stencil_status stencil_plan_schedule_of(stencil_plan_t plan, int64_t tau, const int64_t* s,
+                                        int64_t* sched) {
+  clear_error();
+  Plan* p = as_plan(plan);
+  if (!p || !s || !sched) return fail(STENCIL_E_INVALID, "stencil_plan_schedule_of: bad arguments");
+  if (!schedule_of(*p, tau, s, sched))
+    return fail(STENCIL_E_INVALID, "stencil_plan_schedule_of: point not covered (schedule bug)");
+  return STENCIL_OK;
+}
+
+}  // extern "C"

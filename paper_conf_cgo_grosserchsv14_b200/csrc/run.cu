@@ -1,0 +1,249 @@
+// run.cu -- the host driver (a7): stencil_run.
+//
+// "The T dimension is mapped to the host code, where it takes the form of a for loop
+// repeatedly iterating over two CUDA kernels -- one kernel for p = 0 and the other one for
+// p = 1" (Sec. 4.1).  Each launch-table entry becomes one kernel launch
+// on the caller's stream; the grid is the S0 range of that (T, p).
+#include <cstring>
+
+#include <cuda_runtime.h>
+
+#include "internal.h"
+#include "kernels/launch.h"
+
+namespace hexs {
+
+static stencil_status cuda_fail(cudaError_t e, const char* where) {
+  return fail(STENCIL_E_CUDA, std::string(where) + ": " + cudaGetErrorString(e));
+}
+
+#define HEXS_CUDA(call, where)                    \
+  do {                                            \
+    cudaError_t e_ = (call);                      \
+    if (e_ != cudaSuccess) return cuda_fail(e_, where); \
+  } while (0)
+
+static void fill_generic(const Plan& p, const Launch& l, GenericArgs& g) {
+  const Desc& d = p.desc;
+  g.dims = d.dims;
+  g.hd = p.hd;
+  g.ncls = p.ncls;
+  for (int q = 0; q < 3; ++q) g.N[q] = q < d.dims ? d.ext[q] : 1;
+  g.st[d.dims - 1] = 1;
+  for (int q = d.dims - 2; q >= 0; --q) g.st[q] = g.st[q + 1] * d.ext[q + 1];
+  for (int q = 0; q < 2; ++q) {
+    g.cls[q] = p.cls[q];
+    g.dcls[q] = p.dcls[q];
+    g.w[q] = p.w[q];
+    g.Slo[q] = l.Slo[q];
+    g.Shi[q] = l.Shi[q];
+  }
+  g.tau0 = l.tau0;
+  g.a_lo = l.a_lo;
+  g.a_hi = l.a_hi;
+  g.S0_lo = l.S0_lo;
+  g.row_off = l.row_off;
+  g.W = p.W;
+  g.k0 = d.coef[0];
+  g.k1 = d.coef[1];
+  for (int a = 0; a < p.H; ++a) {
+    g.lo[a] = p.lo[a];
+    g.hi[a] = p.hi[a];
+  }
+}
+
+Plan::~Plan() {
+  for (void* e : prof_events)
+    if (e) cudaEventDestroy(static_cast<cudaEvent_t>(e));
+}
+
+static int64_t launches_per_run(const Plan& p) {
+  return p.executor == EXEC_NAIVE ? p.tau_levels : (int64_t)p.launches.size();
+}
+
+stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* stream_) {
+  const Desc& d = p.desc;
+  // optional per-launch event pairs (stencil_plan_profile)
+  cudaEvent_t* ev = nullptr;
+  if (p.prof_runs > 0 && p.prof_used < p.prof_runs) {
+    ev = reinterpret_cast<cudaEvent_t*>(p.prof_events.data()) + (size_t)p.prof_used * 2 * launches_per_run(p);
+    p.prof_used++;
+  }
+  int64_t li = 0;
+  auto ev_begin = [&](cudaStream_t st) {
+    if (ev) cudaEventRecord(ev[2 * li], st);
+  };
+  auto ev_end = [&](cudaStream_t st) {
+    if (ev) cudaEventRecord(ev[2 * li + 1], st);
+    ++li;
+  };
+  cudaStream_t s = static_cast<cudaStream_t>(stream_);
+  const size_t bytes = (size_t)d.points() * d.elem();
+  int dev = -1;
+  HEXS_CUDA(cudaGetDevice(&dev), "stencil_run: no CUDA device");
+  HEXS_CUDA(cudaGetLastError(), "stencil_run: pending CUDA error");
+
+  for (int f = 0; f < d.nfields; ++f) {
+    if (!in[f] || !out[f]) return fail(STENCIL_E_INVALID, "stencil_run: NULL field pointer");
+    if ((reinterpret_cast<uintptr_t>(in[f]) | reinterpret_cast<uintptr_t>(out[f])) % 16)
+      return fail(STENCIL_E_INVALID, "stencil_run: field pointers must be 16-B aligned");
+    if (in[f] != out[f])
+      HEXS_CUDA(cudaMemcpyAsync(out[f], in[f], bytes, cudaMemcpyDeviceToDevice, s), "stencil_run: copy in->out");
+  }
+  if (p.T_steps == 0) return STENCIL_OK;
+
+  void* buf[2] = {out[0], p.ws};
+  if (d.pingpong) {
+    if (!p.ws || p.ws_size < p.ws_bytes)
+      return fail(STENCIL_E_INVALID, "stencil_run: workspace not set (stencil_plan_set_workspace)");
+    // both ping-pong buffers start as `in`, so Dirichlet cells are valid in either parity
+    HEXS_CUDA(cudaMemcpyAsync(p.ws, out[0], bytes, cudaMemcpyDeviceToDevice, s), "stencil_run: init workspace");
+  }
+
+  if (p.executor == EXEC_NAIVE) {
+    NaiveArgs a{};
+    for (int q = 0; q < 3; ++q) a.N[q] = q < d.dims ? d.ext[q] : 1;
+    a.k0 = d.coef[0];
+    a.k1 = d.coef[1];
+    for (int f = 0; f < d.nfields; ++f) a.f[f] = out[f];
+    for (int64_t tau = 0; tau < p.tau_levels; ++tau) {
+      a.src = buf[tau & 1];
+      a.dst = buf[(tau + 1) & 1];
+      a.stmt = (int)(tau % (int64_t)d.stmts.size());
+      ev_begin(s);
+      HEXS_CUDA(launch_naive(d.kind, d.dtype, d.dims, a, s), "stencil_run: naive kernel launch");
+      ev_end(s);
+    }
+  } else {
+    for (const Launch& l : p.launches) {
+      const int a_final = (l.tau0 + l.a_hi + 1 == p.tau_levels) ? l.a_hi : -1;
+      const int64_t grid64 = l.S0_hi - l.S0_lo + 1;
+      if (grid64 > INT32_MAX) return fail(STENCIL_E_UNSUPPORTED, "stencil_run: grid too large");
+      const int grid = (int)grid64;
+      ev_begin(s);
+      if (p.executor == EXEC_FAST2D) {
+        Fast2DArgs a{};
+        a.buf[0] = buf[0];
+        a.buf[1] = buf[1];
+        a.N0 = d.ext[0];
+        a.N1 = d.ext[1];
+        a.tau0 = l.tau0;
+        a.a_lo = l.a_lo;
+        a.a_hi = l.a_hi;
+        a.a_final = a_final;
+        a.S0_lo = l.S0_lo;
+        a.row_off = l.row_off;
+        a.W = p.W;
+        a.k0 = d.coef[0];
+        a.k1 = d.coef[1];
+        HEXS_CUDA(launch_fast2d(p.variant, a, grid, s), "stencil_run: fast2d kernel launch");
+      } else if (p.executor == EXEC_FDTD) {
+        FdtdArgs a{};
+        for (int f = 0; f < 3; ++f) a.f[f] = out[f];
+        a.N0 = d.ext[0];
+        a.N1 = d.ext[1];
+        a.tau0 = l.tau0;
+        a.a_lo = l.a_lo;
+        a.a_hi = l.a_hi;
+        a.a_final = a_final;
+        a.S0_lo = l.S0_lo;
+        a.row_off = l.row_off;
+        a.W = p.W;
+        a.k0 = d.coef[0];
+        a.k1 = d.coef[1];
+        HEXS_CUDA(launch_fdtd(p.variant, a, grid, s), "stencil_run: fdtd kernel launch");
+      } else if (p.executor == EXEC_FAST3D) {
+        Fast3DArgs a{};
+        a.buf[0] = buf[0];
+        a.buf[1] = buf[1];
+        a.N0 = d.ext[0];
+        a.N1 = d.ext[1];
+        a.N2 = d.ext[2];
+        a.tau0 = l.tau0;
+        a.a_lo = l.a_lo;
+        a.a_hi = l.a_hi;
+        a.a_final = a_final;
+        a.S0_lo = l.S0_lo;
+        a.row_off = l.row_off;
+        a.W = p.W;
+        a.k0 = d.coef[0];
+        a.k1 = d.coef[1];
+        HEXS_CUDA(launch_fast3d(p.variant, a, grid, s), "stencil_run: fast3d kernel launch");
+      } else {
+        GenericArgs g{};
+        if (d.pingpong) {
+          g.f[0] = buf[0];
+          g.f[1] = buf[1];
+        } else {
+          for (int f = 0; f < 3; ++f) g.f[f] = out[f];
+        }
+        fill_generic(p, l, g);
+        HEXS_CUDA(launch_generic(d.kind, d.dtype, g, grid, s), "stencil_run: generic kernel launch");
+      }
+      ev_end(s);
+    }
+  }
+  // level T_steps lives in buffer T_steps % 2
+  if (d.pingpong && (p.tau_levels & 1))
+    HEXS_CUDA(cudaMemcpyAsync(out[0], p.ws, bytes, cudaMemcpyDeviceToDevice, s), "stencil_run: copy result");
+  return STENCIL_OK;
+}
+
+}  // namespace hexs
+
+using namespace hexs;
+
+extern "C" stencil_status stencil_run(stencil_plan_t plan, const void* const* in, void* const* out,
+                                      int64_t T_steps, void* stream) {
+  clear_error();
+  Plan* p = reinterpret_cast<Plan*>(plan);
+  if (!p || p->magic != kPlanMagic) return fail(STENCIL_E_INVALID, "stencil_run: bad plan");
+  if (!in || !out) return fail(STENCIL_E_INVALID, "stencil_run: in/out is NULL");
+  if (T_steps != p->T_steps) return fail(STENCIL_E_INVALID, "stencil_run: T_steps differs from the plan's");
+  return run_plan(*p, in, out, stream);
+}
+
+extern "C" stencil_status stencil_plan_profile(stencil_plan_t plan, int max_runs) {
+  clear_error();
+  Plan* p = reinterpret_cast<Plan*>(plan);
+  if (!p || p->magic != kPlanMagic || max_runs < 0) return fail(STENCIL_E_INVALID, "stencil_plan_profile: bad arguments");
+  for (void* e : p->prof_events)
+    if (e) cudaEventDestroy(static_cast<cudaEvent_t>(e));
+  p->prof_events.clear();
+  p->prof_runs = 0;
+  p->prof_used = 0;
+  if (max_runs == 0) return STENCIL_OK;
+  const size_t n = (size_t)max_runs * 2 * launches_per_run(*p);
+  p->prof_events.assign(n, nullptr);
+  for (size_t i = 0; i < n; ++i) {
+    cudaEvent_t e;
+    cudaError_t r = cudaEventCreate(&e);
+    if (r != cudaSuccess) return cuda_fail(r, "stencil_plan_profile: cudaEventCreate");
+    p->prof_events[i] = e;
+  }
+  p->prof_runs = max_runs;
+  return STENCIL_OK;
+}
+
+extern "C" stencil_status stencil_plan_profile_read(stencil_plan_t plan, double* kernel_ms, int64_t* launches,
+                                                    double* max_launch_ms) {
+  clear_error();
+  Plan* p = reinterpret_cast<Plan*>(plan);
+  if (!p || p->magic != kPlanMagic || !kernel_ms || !launches || !max_launch_ms)
+    return fail(STENCIL_E_INVALID, "stencil_plan_profile_read: bad arguments");
+  const int64_t n = (int64_t)p->prof_used * launches_per_run(*p);
+  double total = 0, mx = 0;
+  cudaEvent_t* ev = reinterpret_cast<cudaEvent_t*>(p->prof_events.data());
+  for (int64_t i = 0; i < n; ++i) {
+    HEXS_CUDA(cudaEventSynchronize(ev[2 * i + 1]), "stencil_plan_profile_read: sync");
+    float ms = 0;
+    HEXS_CUDA(cudaEventElapsedTime(&ms, ev[2 * i], ev[2 * i + 1]), "stencil_plan_profile_read: elapsed");
+    total += ms;
+    if (ms > mx) mx = ms;
+  }
+  *kernel_ms = total;
+  *launches = n;
+  *max_launch_ms = mx;
+  p->prof_used = 0;
+  return STENCIL_OK;
+}

@@ -1,0 +1,147 @@
+"""GPU parity: the CUDA path (through the C ABI) against the CPU oracle, element by element
+on the same seeded inputs.  Built with --fmad=false and IEEE div/sqrt, the kernels evaluate
+the oracle's expression tree exactly, so the bar is bit-exact equality for every class and
+both precisions (BASELINE.json north star: "bit-exactly when both are built with FMA
+contraction off and the same per-point expression order")."""
+import numpy as np
+import pytest
+
+import oracle
+import stencil_inputs
+
+torch = pytest.importorskip("torch")
+pytestmark = pytest.mark.gpu
+
+from paper_conf_cgo_grosserchsv14_b200 import Plan, Stencil  # noqa: E402
+
+
+def _gpu_run(kind, grid, T, dtype, **tile):
+    st = Stencil(kind, grid.shape, dtype=dtype)
+    plan = Plan(st, T, **tile)
+    x = torch.from_numpy(grid).cuda()
+    out = plan.run(x)
+    torch.cuda.synchronize()
+    return out.cpu().numpy(), plan
+
+
+def _gpu_fdtd(fields, T, dtype, **tile):
+    st = Stencil("fdtd2d", fields[0].shape, dtype=dtype)
+    plan = Plan(st, T, **tile)
+    xs = [torch.from_numpy(f).cuda() for f in fields]
+    outs = plan.run(xs)
+    torch.cuda.synchronize()
+    return [o.cpu().numpy() for o in outs], plan
+
+
+def assert_bitexact(got, exp, what=""):
+    if not np.array_equal(got, exp):
+        diff = np.argwhere(got != exp)
+        i = tuple(diff[0])
+        raise AssertionError(f"{what}: {len(diff)} mismatches, first at {i}: got {got[i]!r} want {exp[i]!r}")
+
+
+KIND2D = ["jacobi2d5", "star2d5", "box2d9", "gradient2d"]
+KIND3D = ["star3d7", "gradient3d", "box3d27"]
+
+
+@pytest.mark.parametrize("kind", KIND2D)
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("executor", ["auto", "generic", "naive"])
+def test_2d_small_ragged(kind, dtype, executor):
+    """256x256 T=32 (configs[0]) and a ragged 131x1037 grid, T not a multiple of 2h+2."""
+    for shape, T, seed in [((256, 256), 32, 1), ((131, 1037), 13, 2)]:
+        g = stencil_inputs.uniform(shape, seed=seed, dtype=dtype)
+        got, plan = _gpu_run(kind, g, T, dtype, executor=executor)
+        assert_bitexact(got, oracle.run(kind, g, T), f"{kind} {dtype.__name__} {executor} {shape}")
+
+
+@pytest.mark.parametrize("h,w0", [(3, 10), (1, 3), (3, 7), (3, 15), (5, 8)])
+def test_fast2d_tiles_multi_chunk(h, w0):
+    """Every compiled star2d5 tile on grids spanning several super-chunks, aligned and
+    unaligned rows, with hexagons cut by the domain and by t = 0 / t = T."""
+    for shape, T in [((300, 2052), 23), ((97, 1601), 11), ((64, 515), 2 * h + 2)]:
+        g = stencil_inputs.uniform(shape, seed=3)
+        got, plan = _gpu_run("star2d5", g, T, np.float32, h=h, w0=w0)
+        assert plan.info["fast_kernel"] == 1
+        assert_bitexact(got, oracle.run("star2d5", g, T), f"h={h} w0={w0} {shape} T={T}")
+
+
+@pytest.mark.parametrize("kind", ["jacobi2d5", "box2d9"])
+def test_fast2d_other_tiles(kind):
+    h, w0 = (1, 3) if kind == "jacobi2d5" else (3, 7)
+    g = stencil_inputs.uniform((200, 1300), seed=6)
+    got, plan = _gpu_run(kind, g, 17, np.float32, h=h, w0=w0)
+    assert plan.info["fast_kernel"] == 1
+    assert_bitexact(got, oracle.run(kind, g, 17), kind)
+
+
+def test_2d_edge_cases():
+    g = stencil_inputs.uniform((37, 41), seed=8)
+    for T in (0, 1, 2, 7, 8, 9):
+        got, _ = _gpu_run("star2d5", g, T, np.float32)
+        assert_bitexact(got, oracle.run("star2d5", g, T), f"T={T}")
+    # minimal grid and a single interior row / column
+    for shape in [(3, 3), (3, 700), (700, 3), (4, 5)]:
+        g = stencil_inputs.uniform(shape, seed=9)
+        got, _ = _gpu_run("box2d9", g, 10, np.float32)
+        assert_bitexact(got, oracle.run("box2d9", g, 10), f"{shape}")
+
+
+def test_in_place_alias():
+    g = stencil_inputs.uniform((150, 600), seed=10)
+    st = Stencil("star2d5", g.shape)
+    plan = Plan(st, 21)
+    x = torch.from_numpy(g).cuda()
+    plan.run(x, out=x)
+    torch.cuda.synchronize()
+    assert_bitexact(x.cpu().numpy(), oracle.run("star2d5", g, 21), "in place")
+
+
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("executor", ["auto", "generic", "naive"])
+def test_fdtd(dtype, executor):
+    for shape, T in [((64, 80), 9), ((101, 257), 17)]:
+        f = stencil_inputs.fields(shape, seed=20, n=3, dtype=dtype)
+        got, _ = _gpu_fdtd(f, T, dtype, executor=executor)
+        exp = oracle.fdtd(*f, T)
+        for name, a, b in zip(("ex", "ey", "hz"), got, exp):
+            assert_bitexact(a, b, f"fdtd {name} {executor} {shape}")
+
+
+@pytest.mark.parametrize("h,w0", [(2, 0), (5, 3), (3, 1)])
+def test_fdtd_tiles(h, w0):
+    f = stencil_inputs.fields((90, 70), seed=21, n=3)
+    got, _ = _gpu_fdtd(f, 11, np.float32, h=h, w0=w0)
+    exp = oracle.fdtd(*f, 11)
+    for a, b in zip(got, exp):
+        assert_bitexact(a, b, f"fdtd h={h} w0={w0}")
+
+
+@pytest.mark.parametrize("kind", KIND3D)
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("executor", ["auto", "generic", "naive"])
+def test_3d(kind, dtype, executor):
+    for shape, T in [((34, 29, 67), 7), ((20, 40, 33), 12)]:
+        g = stencil_inputs.uniform(shape, seed=30, dtype=dtype)
+        got, _ = _gpu_run(kind, g, T, dtype, executor=executor)
+        assert_bitexact(got, oracle.run(kind, g, T), f"{kind} {executor} {shape}")
+
+
+def test_constant_field_full_size_property():
+    """Any size: a constant field 1.0 is a fixpoint of star2d5 (coefficients sum to 1)."""
+    g = np.ones((8192, 8192), np.float32)
+    got, _ = _gpu_run("star2d5", g, 16, np.float32)
+    assert np.all(got == 1)
+
+
+@pytest.mark.slow
+@pytest.mark.parametrize("kind", ["star2d5", "box2d9"])
+def test_full_size_sampled(kind):
+    """configs[1] (8192^2, T=512) in the bench's launch configuration, checked at sampled
+    points (including next to the boundary) with the oracle's dependence-cone sampler."""
+    N, T = 8192, 512
+    g = stencil_inputs.uniform((N, N), seed=0)
+    got, plan = _gpu_run(kind, g, T, np.float32)
+    pts = np.array([[1, 1], [1, N - 2], [N - 2, 1], [N // 2, N // 2], [4097, 17], [1000, 8190]])
+    exp = oracle.points(kind, g, T, pts)
+    assert np.array_equal(got[tuple(pts.T)], exp)
