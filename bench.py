@@ -202,7 +202,11 @@ def run_gpu(args, cfg):
     dev = torch.device("cuda", local)
     fields = make_inputs(kind, ext)
     st = Stencil(kind, ext)
-    plan = Plan(st, T)
+    tile = {}
+    if args.tile:
+        h, w0 = (int(x) for x in args.tile.split(","))
+        tile = {"h": h, "w0": w0}
+    plan = Plan(st, T, **tile)
     info = plan.info
     host = [torch.from_numpy(f).pin_memory() for f in fields]
     xin = [h.to(dev) for h in host]
@@ -300,6 +304,7 @@ def main():
     ap.add_argument("--config", default="heat2d5", choices=sorted(CONFIGS))
     ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
     ap.add_argument("--no-cpu", action="store_true", help="skip the CPU oracle baseline")
+    ap.add_argument("--tile", default="", help="h,w0 override (tuning)")
     args = ap.parse_args()
     args.warmup = max(3, args.warmup)
     if args.impl == "reference":

@@ -19,28 +19,47 @@ HEXS_FAST2D_VARIANTS(HEXS_SEL)
 #define HEXS_CAT(a, b) HEXS_CAT2(a, b)
 using KSel = Sel<HEXS_VARIANT>::K;
 
-#ifndef HEXS_MINB
-#define HEXS_MINB KSel::MINB
-#endif
-
-// Full-time hexagons (every launch except the first and last ones of a run).
-__global__ void __launch_bounds__(KSel::NT, HEXS_MINB)
+// Full-time hexagons on 16-B aligned rows: TMA-staged In rows (the hot kernel).
+__global__ void __launch_bounds__(KSel::NT, KSel::MINB)
 HEXS_CAT(fast2d_kernel_v, HEXS_VARIANT)(const __grid_constant__ Fast2DArgs g) {
-  __shared__ KSel::Smem sm;
-  KSel::template run<false>(g, sm);
+  extern __shared__ __align__(16) unsigned char smem_raw[];
+  KSel::run_tma(g, *reinterpret_cast<KSel::Smem*>(smem_raw));
+}
+// Full-time hexagons on unaligned rows (direct loads).
+__global__ void __launch_bounds__(KSel::NT, 1)
+HEXS_CAT(fast2d_kernel_unaligned_v, HEXS_VARIANT)(const __grid_constant__ Fast2DArgs g) {
+  extern __shared__ __align__(16) unsigned char smem_raw[];
+  KSel::template run_direct<false>(g, *reinterpret_cast<KSel::Smem*>(smem_raw));
 }
 // Hexagons cut by t = 0 or t = T_steps (levels outside [a_lo, a_hi] skipped).
 __global__ void __launch_bounds__(KSel::NT, 1)
 HEXS_CAT(fast2d_kernel_tcut_v, HEXS_VARIANT)(const __grid_constant__ Fast2DArgs g) {
-  __shared__ KSel::Smem sm;
-  KSel::template run<true>(g, sm);
+  extern __shared__ __align__(16) unsigned char smem_raw[];
+  KSel::template run_direct<true>(g, *reinterpret_cast<KSel::Smem*>(smem_raw));
 }
 
 cudaError_t HEXS_CAT(launch_fast2d_v, HEXS_VARIANT)(const Fast2DArgs& a, int grid, cudaStream_t s) {
+  static bool attr_set = false;
+  const int smem = (int)sizeof(KSel::Smem);
+  if (!attr_set) {
+    cudaError_t e = cudaFuncSetAttribute(HEXS_CAT(fast2d_kernel_v, HEXS_VARIANT),
+                                         cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+    if (e == cudaSuccess)
+      e = cudaFuncSetAttribute(HEXS_CAT(fast2d_kernel_unaligned_v, HEXS_VARIANT),
+                               cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+    if (e == cudaSuccess)
+      e = cudaFuncSetAttribute(HEXS_CAT(fast2d_kernel_tcut_v, HEXS_VARIANT),
+                               cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+    if (e != cudaSuccess) return e;
+    attr_set = true;
+  }
+  const bool aligned = ((a.N1 * (int64_t)sizeof(KSel::Elem)) % 16) == 0;
   if (a.a_lo > 0 || a.a_hi < KSel::L - 1)
-    HEXS_CAT(fast2d_kernel_tcut_v, HEXS_VARIANT)<<<grid, KSel::NT, 0, s>>>(a);
+    HEXS_CAT(fast2d_kernel_tcut_v, HEXS_VARIANT)<<<grid, KSel::NT, smem, s>>>(a);
+  else if (aligned)
+    HEXS_CAT(fast2d_kernel_v, HEXS_VARIANT)<<<grid, KSel::NT, smem, s>>>(a);
   else
-    HEXS_CAT(fast2d_kernel_v, HEXS_VARIANT)<<<grid, KSel::NT, 0, s>>>(a);
+    HEXS_CAT(fast2d_kernel_unaligned_v, HEXS_VARIANT)<<<grid, KSel::NT, smem, s>>>(a);
   return cudaGetLastError();
 }
 

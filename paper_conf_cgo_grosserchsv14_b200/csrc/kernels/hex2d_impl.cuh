@@ -20,9 +20,13 @@
 //     row and the slanted-edge inputs) and Out set (w0+4h+3 values per column: the slanted
 //     upper edges and the top row), plus every value of the final time level -- the
 //     interleaved copy-out of Sec. 4.2.1;
+//   * the In rows of the NEXT super-chunk are staged into shared memory by 1-D bulk TMA
+//     copies (one per row, 16-B aligned windows -- the aligned loads of Sec. 4.2.3,
+//     PAPER.md:749-767), refilled level by level as soon as the current chunk has consumed
+//     them and tracked by one mbarrier per level, so no warp waits on HBM latency;
 //   * the level loop and the row loop are fully unrolled from the compile-time hexagon
 //     shape (constraint-based unrolling, Sec. 4.3.2); full tiles run the
-//     branch-free instantiation, tiles cut by the domain run the predicated one
+//     branch-free instantiation, tiles cut by the domain run predicated ones
 //     (full/partial separation, Sec. 4.3.1).
 #pragma once
 #include <cstdint>
@@ -30,6 +34,7 @@
 
 #include "../stencil_ops.cuh"
 #include "launch.h"
+#include "tma.cuh"
 
 namespace hexs {
 namespace fast2d {
@@ -61,6 +66,7 @@ __device__ __forceinline__ T apply(const T (&x)[3][3], const Coef<T>& k) {
 
 template <typename T, int KIND, int H, int W0, int NW>
 struct Kernel {
+  using Elem = T;
   static constexpr int V = VecInfo<T>::V;
   static constexpr int VB = VecInfo<T>::VB;
   static constexpr int L = 2 * H + 2;        // levels per hexagon
@@ -68,27 +74,47 @@ struct Kernel {
   static constexpr int Q = R + 2;            // register rows q = b + 1, b in [-1, R]
   static constexpr int NT = NW * 32;
   static constexpr int C = NT * V;           // super-chunk width (classical tile w1)
-  static constexpr int HALO = 2;             // two left-halo columns per row
   static constexpr int MINB = sizeof(T) == 8 ? 2 : 3;  // resident CTAs/SM the register budget targets
+  static constexpr int NIN = W0 + 4 * H + 5; // In rows per chunk (= In values per column)
+  static constexpr int SW = C + 8;           // staged row width (elements), 16-B granular
 
   struct Smem {
-    T tail[2][L][NW][Q][2];  // [chunk parity][level][warp][row][2 last columns]
+    uint64_t mbar[L];                 // one transaction barrier per level's In rows
+    T tail[2][L][NW][Q][2];           // [chunk parity][level][warp][row][2 last columns]
+    alignas(16) T inrows[NIN][SW];    // In rows of the current chunk (TMA-staged)
   };
 
-  // kind of register row q at level a
-  __host__ __device__ static constexpr bool is_in_row(int a, int q) {   // loaded from global at level a
-    const int b = q - 1;
-    if (a == 0) return b >= lo_row(H, W0, 0) - 1 && b <= hi_row(H, W0, 0) + 1;
-    if (a <= H) return b == lo_row(H, W0, a) - 1 || b == lo_row(H, W0, a) ||
-                       b == hi_row(H, W0, a) || b == hi_row(H, W0, a) + 1;
-    if (a == H + 1) return b == -1 || b == R;
+  // ---- compile-time hexagon shape ----
+  __host__ __device__ static constexpr int n_in(int a) {
+    return a == 0 ? W0 + 3 : (a <= H ? 4 : (a == H + 1 ? 2 : 0));
+  }
+  __host__ __device__ static constexpr int slot_base(int a) {
+    return a == 0 ? 0 : (a <= H ? W0 + 3 + 4 * (a - 1) : W0 + 3 + 4 * H);
+  }
+  // local row b of the i-th In row of level a
+  __host__ __device__ static constexpr int in_row_b(int a, int i) {
+    if (a == 0) return lo_row(H, W0, 0) - 1 + i;
+    if (a <= H) {
+      const int lo = lo_row(H, W0, a), hi = hi_row(H, W0, a);
+      return i == 0 ? lo - 1 : (i == 1 ? lo : (i == 2 ? hi : hi + 1));
+    }
+    return i == 0 ? -1 : R;
+  }
+  __host__ __device__ static constexpr bool is_in_row(int a, int q) {   // loaded at level a
+    for (int i = 0; i < n_in(a); ++i)
+      if (in_row_b(a, i) == q - 1) return true;
     return false;
   }
-  __host__ __device__ static constexpr bool is_input_row(int a, int q) {  // any input row of level a
+  __host__ __device__ static constexpr int in_slot(int a, int q) {
+    for (int i = 0; i < n_in(a); ++i)
+      if (in_row_b(a, i) == q - 1) return slot_base(a) + i;
+    return -1;
+  }
+  __host__ __device__ static constexpr bool is_input_row(int a, int q) {
     const int b = q - 1;
     return b >= lo_row(H, W0, a) - 1 && b <= hi_row(H, W0, a) + 1;
   }
-  __host__ __device__ static constexpr bool is_out_row(int a, int q) {  // in the Out set (stored) at level a
+  __host__ __device__ static constexpr bool is_out_row(int a, int q) {  // Out set (stored) at level a
     const int b = q - 1, lo = lo_row(H, W0, a), hi = hi_row(H, W0, a);
     if (b < lo || b > hi) return false;
     if (a < H) return false;
@@ -96,52 +122,52 @@ struct Kernel {
     if (a < L - 1) return b <= lo + 1 || b >= hi - 1;
     return true;
   }
-  __host__ __device__ static constexpr bool is_comp_row(int a, int q) {
-    const int b = q - 1;
-    return b >= lo_row(H, W0, a) && b <= hi_row(H, W0, a);
+  // first column of the staged window of level a (16-B aligned: k*C and C are multiples of VB)
+  __host__ __device__ static constexpr int win_shift(int a) {  // window start = k*C - win_shift(a)
+    return a + 1 + (((-a - 1) % VB + VB) % VB);
   }
 
-  // Load V+2 consecutive elements starting at column `start` (= thread's first halo
-  // column) of global row `row` into dst[0..V+1].  aligned: row pitch is 16-B granular so
-  // aligned 16-B block loads are legal; the misalignment (start mod VB) is the
-  // compile-time constant M.
-  template <int M, bool PART>
-  static __device__ __forceinline__ void load_window(const T* __restrict__ src, int64_t N1, int64_t row,
-                                                     int start, bool aligned, T (&dst)[V + 2]) {
-    const T* rp = src + row * N1;
-    if (aligned && (!PART || (start - M >= 0 && start - M + 3 * VB <= N1))) {
-      constexpr int NB = (M + V + 2 + VB - 1) / VB;  // 16-B blocks covering [M, M+V+2)
-      T blk[NB * VB];
-      const T* bp = rp + (start - M);
-#pragma unroll
-      for (int i = 0; i < NB; ++i) {
-        if constexpr (VB == 4) {
-          const float4 v = *(reinterpret_cast<const float4*>(bp) + i);
-          blk[4 * i] = v.x; blk[4 * i + 1] = v.y; blk[4 * i + 2] = v.z; blk[4 * i + 3] = v.w;
-        } else {
-          const double2 v = *(reinterpret_cast<const double2*>(bp) + i);
-          blk[2 * i] = v.x; blk[2 * i + 1] = v.y;
-        }
-      }
-#pragma unroll
-      for (int i = 0; i < V + 2; ++i) dst[i] = blk[M + i];
-    } else {
-#pragma unroll
-      for (int i = 0; i < V + 2; ++i) {
-        int64_t col = (int64_t)start + i;
-        if constexpr (PART) col = col < 0 ? 0 : (col >= N1 ? N1 - 1 : col);
-        dst[i] = rp[col];
-      }
+  // ---- producer: TMA the In rows of (chunk k, level a) into their slots (thread 0) ----
+  static __device__ __forceinline__ void issue_level(const Fast2DArgs& g, Smem& sm, int64_t k, int a,
+                                                     int64_t i0) {
+    const int na = n_in(a);
+    if (na == 0) return;
+    const T* src = static_cast<const T*>(g.buf[(g.tau0 + a) & 1]);  // input level tau0 + a
+    const int64_t N0 = g.N0, N1 = g.N1;
+    const int64_t c0 = k * C - win_shift(a);
+    const int64_t lo_c = c0 < 0 ? 0 : c0;
+    const int64_t hi_c = (c0 + SW) > N1 ? N1 : (c0 + SW);
+    const uint32_t bytes = hi_c > lo_c ? (uint32_t)((hi_c - lo_c) * sizeof(T)) : 0u;
+    mbar_arrive_expect_tx(&sm.mbar[a], bytes * na);
+    if (bytes == 0) return;
+    for (int i = 0; i < na; ++i) {
+      int64_t row = i0 + in_row_b(a, i);
+      row = row < 0 ? 0 : (row >= N0 ? N0 - 1 : row);
+      tma_load_1d(&sm.inrows[slot_base(a) + i][lo_c - c0], src + row * N1 + lo_c, bytes, &sm.mbar[a]);
     }
   }
 
-  // One super-chunk: all levels a in [a_lo, a_hi] of columns [k*C - a, k*C - a + C).
-  // PART: tile cut by the domain (predicated points); TCUT: tile cut in time (levels
-  // outside [a_lo, a_hi] are skipped at run time).  Full tiles run <false, false>, which is
-  // free of any run-time level control so every register row has a static live range.
-  template <bool PART, bool TCUT>
-  static __device__ __forceinline__ void chunk(const Fast2DArgs& g, Smem& sm, int64_t k, int64_t i0,
-                                               int a_final, bool aligned, const Coef<T>& cf) {
+  // Direct (non-TMA) load of V+2 consecutive elements starting at column `start` of global
+  // row `row` (unaligned rows or time-cut tiles); clamped into the grid.
+  static __device__ __forceinline__ void load_direct(const T* src, int64_t N1, int64_t row, int start,
+                                                     T (&dst)[V + 2]) {
+    const T* rp = src + row * N1;
+#pragma unroll
+    for (int i = 0; i < V + 2; ++i) {
+      int64_t col = (int64_t)start + i;
+      col = col < 0 ? 0 : (col >= N1 ? N1 - 1 : col);
+      dst[i] = rp[col];
+    }
+  }
+
+  // One super-chunk: all levels of columns [k*C - a, k*C - a + C).
+  //   TMA : In rows come from the TMA-staged slots (else direct global loads)
+  //   ROWP: hexagon rows cross the domain's row boundary (per-row uniform predicate)
+  //   COLP: chunk crosses a column boundary (per-element predicate)
+  //   TCUT: tile cut at t = 0 / t = T (levels outside [a_lo, a_hi] skipped at run time)
+  template <bool TMA, bool ROWP, bool COLP, bool TCUT>
+  static __device__ __forceinline__ void chunk(const Fast2DArgs& g, Smem& sm, int64_t k, int64_t K,
+                                               int64_t i0, const Coef<T>& cf) {
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
     const int64_t N0 = g.N0, N1 = g.N1;
     T in[Q][V + 2];  // input array of the current level: [row][halo0, halo1, own V]
@@ -159,28 +185,48 @@ struct Kernel {
       const T* src = static_cast<const T*>(g.buf[tau & 1]);
       T* dst = static_cast<T*>(g.buf[(tau + 1) & 1]);
       const int colbase = (int)k * C - a + tid * V;  // first output column (N1 < 2^30)
-      const int wstart = colbase - 1;                // first input column (halo)
-      constexpr int M = ((-a - 1) % VB + VB) % VB;             // wstart mod VB (k*C, tid*V are multiples of VB)
       const bool first = TCUT ? (a == g.a_lo) : (a == 0);
 
-      // ---- (1) inputs: In rows from global (all input rows at the first level) ----
-#pragma unroll
-      for (int q = 0; q < Q; ++q) {
-        if (!is_input_row(a, q)) continue;
-        if (first || is_in_row(a, q)) {
-          int64_t row = i0 + (q - 1);
-          if constexpr (PART) row = row < 0 ? 0 : (row >= N0 ? N0 - 1 : row);
-          load_window<M, PART>(src, N1, row, wstart, aligned, in[q]);
-        }
+      // ---- (1) the In rows of this level have landed (TMA mode) ----
+      if constexpr (TMA) {
+        static_assert(!TCUT, "TMA staging runs full-time tiles only");
+        if constexpr (n_in(a) > 0) mbar_wait_parity(&sm.mbar[a], (uint32_t)(k & 1));
       }
-      // ---- (2)-(5) rows ascending: left halo just in time, compute, copy out, tail ----
+
+      // ---- (2)-(5) rows ascending: inputs just in time, compute, copy out, tail ----
       const int pw = warp == 0 ? NW - 1 : warp - 1;
       const int pk = warp == 0 ? (int)((k - 1) & 1) : (int)(k & 1);
-      // Left halo of input row q: rows computed at the previous level take the two last
-      // columns of the left lane (shuffle) or, in lane 0, of the previous warp / chunk
-      // (shared-memory tail).  Rows loaded from global already carry their halo.
+      // Input row q of level a, fetched right before its first use (keeps the register
+      // footprint at ~one level of rows): In rows come from the TMA-staged slot (or global
+      // memory) with their two left-halo columns; rows computed at the previous level take
+      // the two last columns of the left lane (shuffle) or, in lane 0, of the previous warp /
+      // chunk (shared-memory tail).
       auto halo = [&](auto q_c) {
         constexpr int q = decltype(q_c)::value;
+        if constexpr (TMA && is_in_row(a, q)) {
+          constexpr int M = win_shift(a) - a - 1;  // window offset of the thread's first input column
+          constexpr int NB = (M + V + 2 + VB - 1) / VB;
+          const T* rowp = &sm.inrows[in_slot(a, q)][tid * V];
+          T blk[NB * VB];
+#pragma unroll
+          for (int i = 0; i < NB; ++i) {
+            if constexpr (VB == 4) {
+              const float4 v4 = reinterpret_cast<const float4*>(rowp)[i];
+              blk[4 * i] = v4.x; blk[4 * i + 1] = v4.y; blk[4 * i + 2] = v4.z; blk[4 * i + 3] = v4.w;
+            } else {
+              const double2 v2 = reinterpret_cast<const double2*>(rowp)[i];
+              blk[2 * i] = v2.x; blk[2 * i + 1] = v2.y;
+            }
+          }
+#pragma unroll
+          for (int i = 0; i < V + 2; ++i) in[q][i] = blk[M + i];
+        } else if constexpr (!TMA && is_input_row(a, q)) {
+          if (first || is_in_row(a, q)) {
+            int64_t row = i0 + (q - 1);
+            row = row < 0 ? 0 : (row >= N0 ? N0 - 1 : row);
+            load_direct(src, N1, row, colbase - 1, in[q]);
+          }
+        }
         if constexpr (is_input_row(a, q) && !is_in_row(a, q) && a > 0) {
           if (!first) {
             T h0 = __shfl_up_sync(0xffffffffu, in[q][V], 1);
@@ -202,14 +248,15 @@ struct Kernel {
 #pragma unroll
       for (int v = 0; v < V; ++v) {
         const int c = colbase + v;
-        colok[v] = !PART || (c >= 1 && c <= (int)N1 - 2);
+        colok[v] = !COLP || (c >= 1 && c <= (int)N1 - 2);
       }
-      const bool fin = TCUT && (a == a_final);
+      const bool fin = TCUT && (a == g.a_final);
+      T* dbase = dst + i0 * N1 + colbase;
       static_for<qlo, qhi + 1>([&](auto q_c) {
         constexpr int q = decltype(q_c)::value;
         halo(std::integral_constant<int, q + 1>{});
         const int64_t row = i0 + (q - 1);
-        const bool rowok = !PART || (row >= 1 && row <= N0 - 2);
+        const bool rowok = !ROWP || (row >= 1 && row <= N0 - 2);
 #pragma unroll
         for (int v = 0; v < V; ++v) {
           T x[3][3];
@@ -218,16 +265,16 @@ struct Kernel {
 #pragma unroll
             for (int c = 0; c < 3; ++c) x[r][c] = in[q - 1 + r][v + c];
           const T val = apply<T, KIND>(x, cf);
-          if constexpr (PART) out[q][v] = (rowok && colok[v]) ? val : in[q][v + 1];
+          if constexpr (ROWP || COLP) out[q][v] = (rowok && colok[v]) ? val : in[q][v + 1];
           else out[q][v] = val;
         }
         // interleaved copy-out of the Out set (every row at the final level)
         if (is_out_row(a, q) || fin) {
-          if (!PART || rowok) {
-            T* rp = dst + row * N1 + colbase;
+          if (rowok) {
+            T* rp = dbase + (int64_t)(q - 1) * N1;
 #pragma unroll
             for (int v = 0; v < V; ++v)
-              if (!PART || colok[v]) rp[v] = out[q][v];
+              if (colok[v]) rp[v] = out[q][v];
           }
         }
         // tail for the next warp / next super-chunk
@@ -239,6 +286,13 @@ struct Kernel {
         }
       });
       __syncthreads();
+      // ---- refill: the consumed slots of level a take chunk k+1's In rows ----
+      if constexpr (TMA && n_in(a) > 0) {
+        if (tid == 0 && k + 1 < K) {
+          fence_proxy_async_smem();
+          issue_level(g, sm, k + 1, a, i0);
+        }
+      }
       // ---- (6) the outputs become the next level's inputs ----
 #pragma unroll
       for (int q = qlo; q <= qhi; ++q)
@@ -247,21 +301,50 @@ struct Kernel {
     });
   }
 
-  template <bool TCUT>
-  static __device__ __forceinline__ void run(const Fast2DArgs& g, Smem& sm) {
+  static __device__ __forceinline__ int64_t n_chunks(const Fast2DArgs& g) {
+    return (g.N1 + L - 2 + C - 1) / C;
+  }
+  static __device__ __forceinline__ bool col_partial(const Fast2DArgs& g, int64_t k) {
+    return (k == 0) || ((k + 1) * C > g.N1 - 1) || (k * C - (L - 1) < 1);
+  }
+
+  // Full-time tiles, 16-B aligned rows: TMA-staged In rows.
+  static __device__ __forceinline__ void run_tma(const Fast2DArgs& g, Smem& sm) {
     const int64_t S0 = g.S0_lo + blockIdx.x;
     const int64_t i0 = S0 * g.W - g.row_off;  // global row of local row b = 0
     const Coef<T> cf{(T)g.k0, (T)g.k1};
-    const int64_t N0 = g.N0, N1 = g.N1;
-    const bool aligned = ((N1 * (int64_t)sizeof(T)) % 16) == 0;
-    const bool rowpart = (i0 - 1 < 1) || (i0 + R > N0 - 2);
-    const int64_t K = (N1 + L - 2 + C - 1) / C;
-    for (int64_t k = 0; k < K; ++k) {
-      const bool colpart = (k == 0) || ((k + 1) * C > N1 - 1) || (k * C - (L - 1) < 1);
-      if constexpr (TCUT) chunk<true, true>(g, sm, k, i0, g.a_final, aligned, cf);
-      else if (rowpart || colpart) chunk<true, false>(g, sm, k, i0, g.a_final, aligned, cf);
-      else chunk<false, false>(g, sm, k, i0, g.a_final, aligned, cf);
+    const bool rowpart = (i0 - 1 < 1) || (i0 + R > g.N0 - 2);
+    const int64_t K = n_chunks(g);
+    if (threadIdx.x == 0) {
+#pragma unroll
+      for (int a = 0; a < L; ++a) mbar_init(&sm.mbar[a], 1);
+      mbar_fence_init();
     }
+    __syncthreads();
+    if (threadIdx.x == 0) {
+#pragma unroll
+      for (int a = 0; a < L; ++a) issue_level(g, sm, 0, a, i0);
+    }
+    for (int64_t k = 0; k < K; ++k) {
+      const bool colpart = col_partial(g, k);
+      if (rowpart) {
+        if (colpart) chunk<true, true, true, false>(g, sm, k, K, i0, cf);
+        else chunk<true, true, false, false>(g, sm, k, K, i0, cf);
+      } else {
+        if (colpart) chunk<true, false, true, false>(g, sm, k, K, i0, cf);
+        else chunk<true, false, false, false>(g, sm, k, K, i0, cf);
+      }
+    }
+  }
+
+  // Unaligned rows (TCUT = false) or time-cut tiles (TCUT = true): direct loads, predicated.
+  template <bool TCUT>
+  static __device__ __forceinline__ void run_direct(const Fast2DArgs& g, Smem& sm) {
+    const int64_t S0 = g.S0_lo + blockIdx.x;
+    const int64_t i0 = S0 * g.W - g.row_off;
+    const Coef<T> cf{(T)g.k0, (T)g.k1};
+    const int64_t K = n_chunks(g);
+    for (int64_t k = 0; k < K; ++k) chunk<false, true, true, TCUT>(g, sm, k, K, i0, cf);
   }
 };
 
