@@ -36,6 +36,10 @@
 #include "launch.h"
 #include "tma.cuh"
 
+#ifndef HEXS_MERGE_ROWP
+#define HEXS_MERGE_ROWP 1
+#endif
+
 namespace hexs {
 namespace fast2d {
 
@@ -327,6 +331,14 @@ struct Kernel {
     }
     for (int64_t k = 0; k < K; ++k) {
       const bool colpart = col_partial(g, k);
+#if HEXS_MERGE_ROWP
+      // One code body for interior and row-partial hexagons (a per-element select on the
+      // row predicate): co-resident CTAs then share the instruction stream instead of
+      // thrashing the instruction cache with two ~70 KB bodies.
+      (void)rowpart;
+      if (colpart) chunk<true, true, true, false>(g, sm, k, K, i0, cf);
+      else chunk<true, true, false, false>(g, sm, k, K, i0, cf);
+#else
       if (rowpart) {
         if (colpart) chunk<true, true, true, false>(g, sm, k, K, i0, cf);
         else chunk<true, true, false, false>(g, sm, k, K, i0, cf);
@@ -334,6 +346,7 @@ struct Kernel {
         if (colpart) chunk<true, false, true, false>(g, sm, k, K, i0, cf);
         else chunk<true, false, false, false>(g, sm, k, K, i0, cf);
       }
+#endif
     }
   }
 
