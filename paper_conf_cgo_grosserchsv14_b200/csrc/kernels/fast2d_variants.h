@@ -1,20 +1,22 @@
 // fast2d_variants.h -- the compiled instantiations of the fast 2D kernel:
 // X(id, dtype_code, T, KIND, h, w0, NW).  Each id is compiled from fast2d_inst.cu with
-// -DHEXS_VARIANT=id into its own object (parallel build).
+// -DHEXS_VARIANT=id into its own object (parallel build).  (3, 7) is the default tile
+// (DESIGN.md "tile selection"); the others serve the tile sweep and the tests.
 #pragma once
 #define HEXS_FAST2D_VARIANTS(X)                  \
-  X(0, 0, float, K_STAR2D5, 3, 10, 4)            \
-  X(1, 0, float, K_JACOBI2D5, 3, 10, 4)          \
-  X(2, 0, float, K_BOX2D9, 3, 10, 4)             \
-  X(3, 0, float, K_GRADIENT2D, 3, 10, 4)         \
-  X(4, 1, double, K_STAR2D5, 3, 10, 4)           \
-  X(5, 1, double, K_JACOBI2D5, 3, 10, 4)         \
-  X(6, 0, float, K_STAR2D5, 1, 3, 4)             \
-  X(7, 0, float, K_STAR2D5, 3, 7, 4)             \
-  X(8, 0, float, K_STAR2D5, 3, 15, 4)            \
-  X(9, 0, float, K_STAR2D5, 5, 8, 4)             \
-  X(10, 0, float, K_BOX2D9, 3, 7, 4)             \
-  X(11, 1, double, K_BOX2D9, 3, 10, 4)           \
-  X(12, 1, double, K_GRADIENT2D, 3, 10, 4)       \
-  X(13, 0, float, K_JACOBI2D5, 1, 3, 4)
-#define HEXS_FAST2D_COUNT 14
+  X(0, 0, float, K_STAR2D5, 3, 7, 4)             \
+  X(1, 0, float, K_JACOBI2D5, 3, 7, 4)           \
+  X(2, 0, float, K_BOX2D9, 3, 7, 4)              \
+  X(3, 0, float, K_GRADIENT2D, 3, 7, 4)          \
+  X(4, 1, double, K_STAR2D5, 3, 7, 4)            \
+  X(5, 1, double, K_JACOBI2D5, 3, 7, 4)          \
+  X(6, 1, double, K_BOX2D9, 3, 7, 4)             \
+  X(7, 1, double, K_GRADIENT2D, 3, 7, 4)         \
+  X(8, 0, float, K_STAR2D5, 1, 3, 4)             \
+  X(9, 0, float, K_STAR2D5, 3, 10, 4)            \
+  X(10, 0, float, K_STAR2D5, 2, 5, 4)            \
+  X(11, 0, float, K_STAR2D5, 3, 5, 4)            \
+  X(12, 0, float, K_STAR2D5, 4, 5, 4)            \
+  X(13, 0, float, K_JACOBI2D5, 1, 3, 4)          \
+  X(14, 0, float, K_BOX2D9, 3, 5, 4)
+#define HEXS_FAST2D_COUNT 15

@@ -55,7 +55,7 @@ def test_2d_small_ragged(kind, dtype, executor):
         assert_bitexact(got, oracle.run(kind, g, T), f"{kind} {dtype.__name__} {executor} {shape}")
 
 
-@pytest.mark.parametrize("h,w0", [(3, 10), (1, 3), (3, 7), (3, 15), (5, 8)])
+@pytest.mark.parametrize("h,w0", [(3, 7), (1, 3), (3, 10), (2, 5), (4, 5)])
 def test_fast2d_tiles_multi_chunk(h, w0):
     """Every compiled star2d5 tile on grids spanning several super-chunks, aligned and
     unaligned rows, with hexagons cut by the domain and by t = 0 / t = T."""
@@ -68,7 +68,7 @@ def test_fast2d_tiles_multi_chunk(h, w0):
 
 @pytest.mark.parametrize("kind", ["jacobi2d5", "box2d9"])
 def test_fast2d_other_tiles(kind):
-    h, w0 = (1, 3) if kind == "jacobi2d5" else (3, 7)
+    h, w0 = (1, 3) if kind == "jacobi2d5" else (3, 5)
     g = stencil_inputs.uniform((200, 1300), seed=6)
     got, plan = _gpu_run(kind, g, 17, np.float32, h=h, w0=w0)
     assert plan.info["fast_kernel"] == 1
