@@ -30,8 +30,10 @@ def _splitmix64(x: np.ndarray) -> np.ndarray:
 
 
 def uniform(shape: Sequence[int], seed: int, dtype=np.float32, out: np.ndarray = None,
-            chunk: int = 1 << 24) -> np.ndarray:
-    """Fill an array of `shape` with the counter-based uniform values of `seed`."""
+            chunk: int = 1 << 24, offset: int = 0) -> np.ndarray:
+    """Fill an array of `shape` with the counter-based uniform values of `seed`; element k
+    of the (flattened) array is the value of linear index offset + k, so a slab of a
+    larger grid can be generated on its own (multi-GPU ranks)."""
     shape = tuple(int(s) for s in shape)
     n = int(np.prod(shape))
     if out is None:
@@ -41,7 +43,7 @@ def uniform(shape: Sequence[int], seed: int, dtype=np.float32, out: np.ndarray =
     with np.errstate(over="ignore"):
         for lo in range(0, n, chunk):
             hi = min(n, lo + chunk)
-            idx = np.arange(lo, hi, dtype=np.uint64)
+            idx = np.arange(lo + offset, hi + offset, dtype=np.uint64)
             z = _splitmix64(idx ^ key)
             flat[lo:hi] = (z >> np.uint64(40)).astype(np.float64) * (2.0 ** -24)
     return out
