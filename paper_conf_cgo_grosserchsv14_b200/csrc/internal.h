@@ -83,6 +83,8 @@ struct Plan {
   int executor = EXEC_GENERIC;
   int variant = 0;  // fast-kernel instantiation id
   int64_t tile_points = 0, tile_in = 0, tile_out = 0;
+  bool wavefront = false;      // generic executor: classical tiles as a dependence wavefront
+  size_t flag_off = 0, counter_off = 0, flag_bytes = 0;  // workspace layout (wavefront)
   size_t ws_bytes = 0;
   void* ws = nullptr;
   size_t ws_size = 0;

@@ -45,35 +45,106 @@ __device__ __forceinline__ void generic_point(const GenericArgs& g, int64_t tau,
   }
 }
 
+// All levels of one classical tile (q1, q2) of hexagon S0.
+template <typename T, int KIND>
+__device__ __forceinline__ void generic_tile(const GenericArgs& g, int64_t S0, int64_t q1, int64_t q2,
+                                             const Coef<T>& k) {
+  const int64_t i0 = S0 * g.W - g.row_off;  // spatial coordinate of local row b = 0
+  const int w1 = g.ncls >= 1 ? g.w[0] : 1, w2 = g.ncls >= 2 ? g.w[1] : 1;
+  for (int a = g.a_lo; a <= g.a_hi; ++a) {  // tile-local time t', sequential
+    const int64_t tau = g.tau0 + a;
+    const int rows = g.hi[a] - g.lo[a] + 1;
+    const int64_t base1 = (g.Slo[0] + q1) * w1 - (int64_t)g.dcls[0] * a;  // eq. (14)
+    const int64_t base2 = (g.Slo[1] + q2) * w2 - (int64_t)g.dcls[1] * a;
+    const int64_t total = (int64_t)rows * w1 * w2;
+    for (int64_t e = threadIdx.x; e < total; e += blockDim.x) {  // s -> threads, cyclic
+      const int x2 = (int)(e % w2);
+      const int64_t r = e / w2;
+      const int x1 = (int)(r % w1);
+      const int b = (int)(r / w1) + g.lo[a];
+      int64_t c[3] = {0, 0, 0};
+      c[g.hd] = i0 + b;
+      if (g.ncls >= 1) c[g.cls[0]] = base1 + x1;
+      if (g.ncls >= 2) c[g.cls[1]] = base2 + x2;
+      generic_point<T, KIND>(g, tau, c, k);
+    }
+    __syncthreads();
+  }
+}
+
 template <typename T, int KIND>
 __global__ void __launch_bounds__(256) generic_kernel(const __grid_constant__ GenericArgs g) {
   const int64_t S0 = g.S0_lo + blockIdx.x;
-  const int64_t i0 = S0 * g.W - g.row_off;  // spatial coordinate of local row b = 0
   const Coef<T> k{(T)g.k0, (T)g.k1};
-  const int w1 = g.ncls >= 1 ? g.w[0] : 1, w2 = g.ncls >= 2 ? g.w[1] : 1;
   const int64_t n1 = g.ncls >= 1 ? g.Shi[0] - g.Slo[0] + 1 : 1;
   const int64_t n2 = g.ncls >= 2 ? g.Shi[1] - g.Slo[1] + 1 : 1;
-  for (int64_t q1 = 0; q1 < n1; ++q1) {      // classical tiles, sequential (Sec. 4.1)
-    for (int64_t q2 = 0; q2 < n2; ++q2) {
-      for (int a = g.a_lo; a <= g.a_hi; ++a) {  // tile-local time t', sequential
-        const int64_t tau = g.tau0 + a;
-        const int rows = g.hi[a] - g.lo[a] + 1;
-        const int64_t base1 = (g.Slo[0] + q1) * w1 - (int64_t)g.dcls[0] * a;  // eq. (14)
-        const int64_t base2 = (g.Slo[1] + q2) * w2 - (int64_t)g.dcls[1] * a;
-        const int64_t total = (int64_t)rows * w1 * w2;
-        for (int64_t e = threadIdx.x; e < total; e += blockDim.x) {  // s -> threads, cyclic
-          const int x2 = (int)(e % w2);
-          const int64_t r = e / w2;
-          const int x1 = (int)(r % w1);
-          const int b = (int)(r / w1) + g.lo[a];
-          int64_t c[3] = {0, 0, 0};
-          c[g.hd] = i0 + b;
-          if (g.ncls >= 1) c[g.cls[0]] = base1 + x1;
-          if (g.ncls >= 2) c[g.cls[1]] = base2 + x2;
-          generic_point<T, KIND>(g, tau, c, k);
+  for (int64_t q1 = 0; q1 < n1; ++q1)      // classical tiles, sequential (Sec. 4.1)
+    for (int64_t q2 = 0; q2 < n2; ++q2) generic_tile<T, KIND>(g, S0, q1, q2, k);
+}
+
+__device__ __forceinline__ int ld_acquire(const int* p) {
+  int v;
+  asm volatile("ld.acquire.gpu.global.b32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
+  return v;
+}
+__device__ __forceinline__ void st_release(int* p, int v) {
+  asm volatile("st.release.gpu.global.b32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
+}
+
+// Wavefront execution: the classical tiles of a hexagon form a 2-D dependence grid
+// ((S1, S2) needs (S1-1, S2) and (S1, S2-1) -- eq. (14)'s skew makes every dependence point
+// to a lower tile index).  Tiles on one anti-diagonal are independent, so a hexagon's
+// classical tiles run concurrently on many SMs instead of sequentially on one (the paper's
+// mapping, Sec. 4.1, leaves S1..Sn sequential; with 148 SMs and ~26-51 hexagons per phase
+// on 512^3 that would idle most of the GPU).  Persistent CTAs fetch items in (diagonal,
+// S0, S1) order; every item waits only for items fetched earlier, so the grid (all CTAs
+// resident) cannot deadlock.
+template <typename T, int KIND>
+__global__ void __launch_bounds__(256) generic_wf_kernel(const __grid_constant__ GenericArgs g) {
+  __shared__ int64_t item_s[3];
+  const Coef<T> k{(T)g.k0, (T)g.k1};
+  const int64_t n1 = g.Shi[0] - g.Slo[0] + 1;
+  const int64_t n2 = g.ncls >= 2 ? g.Shi[1] - g.Slo[1] + 1 : 1;
+  const int64_t ns0 = g.S0_hi - g.S0_lo + 1;
+  const int64_t n_items = ns0 * n1 * n2;
+  while (true) {
+    if (threadIdx.x == 0) {
+      const int64_t it = (int64_t)atomicAdd(g.counter, 1ull);
+      int64_t S0 = -1, q1 = 0, q2 = 0;
+      if (it < n_items) {
+        // decode: anti-diagonal d = q1 + q2 (outer), then S0, then q1
+        int64_t off = 0;
+        for (int64_t d = 0; d < n1 + n2 - 1; ++d) {
+          const int64_t lo1 = d - (n2 - 1) > 0 ? d - (n2 - 1) : 0;
+          const int64_t hi1 = d < n1 - 1 ? d : n1 - 1;
+          const int64_t pairs = hi1 - lo1 + 1;
+          if (it < off + pairs * ns0) {
+            const int64_t r = it - off;
+            S0 = g.S0_lo + r / pairs;
+            q1 = lo1 + r % pairs;
+            q2 = d - q1;
+            break;
+          }
+          off += pairs * ns0;
         }
-        __syncthreads();
+        const int64_t base = (S0 - g.S0_lo) * n1 * n2;
+        if (q1 > 0)
+          while (ld_acquire(g.flags + base + (q1 - 1) * n2 + q2) == 0) __nanosleep(64);
+        if (q2 > 0)
+          while (ld_acquire(g.flags + base + q1 * n2 + q2 - 1) == 0) __nanosleep(64);
+        __threadfence();  // gpu-scope fence: drop stale L1 lines before reading neighbours
       }
+      item_s[0] = S0;
+      item_s[1] = q1;
+      item_s[2] = q2;
+    }
+    __syncthreads();
+    const int64_t S0 = item_s[0], q1 = item_s[1], q2 = item_s[2];
+    if (S0 < 0) break;
+    generic_tile<T, KIND>(g, S0, q1, q2, k);  // ends with __syncthreads
+    if (threadIdx.x == 0) {
+      __threadfence();
+      st_release(g.flags + (S0 - g.S0_lo) * n1 * n2 + q1 * n2 + q2, 1);
     }
   }
 }
@@ -98,18 +169,35 @@ __global__ void __launch_bounds__(256) naive2d_kernel(const T* __restrict__ src,
   }
 }
 
+// 3D naive step: block = 64 (x) x 4 (y) columns marching over a z-strip; the z-neighbours
+// stay in a register queue, the in-plane neighbours come from L1 (shared by the block's
+// lines).  One read of each plane from DRAM per step when L1/L2 absorb the reuse.
+constexpr int kNaive3DStrip = 32;
 template <typename T, int KIND>
 __global__ void __launch_bounds__(256) naive3d_kernel(const T* __restrict__ src, T* __restrict__ dst,
                                                       int64_t N0, int64_t N1, int64_t N2, Coef<T> k) {
-  const int64_t x = 1 + blockIdx.x * (int64_t)blockDim.x + threadIdx.x;
-  const int64_t y = 1 + blockIdx.y;
-  const int64_t z_start = 1 + (int64_t)blockIdx.z * kNaiveStrip;
-  if (x > N2 - 2) return;
-  const int64_t z_end = z_start + kNaiveStrip < N0 - 1 ? z_start + kNaiveStrip : N0 - 1;
+  const int64_t x = 1 + blockIdx.x * 64 + threadIdx.x;
+  const int64_t y = 1 + (int64_t)blockIdx.y * 4 + threadIdx.y;
+  const int64_t z_start = 1 + (int64_t)blockIdx.z * kNaive3DStrip;
+  if (x > N2 - 2 || y > N1 - 2) return;
+  const int64_t z_end = z_start + kNaive3DStrip < N0 - 1 ? z_start + kNaive3DStrip : N0 - 1;
   const int64_t s0 = N1 * N2;
-  for (int64_t z = z_start; z < z_end; ++z) {
-    const int64_t p = z * s0 + y * N2 + x;
-    dst[p] = point_from_memory<T, KIND>(src, p, s0, N2, k);
+  if constexpr (KIND == K_STAR3D7 || KIND == K_GRADIENT3D) {
+    int64_t p = z_start * s0 + y * N2 + x;
+    T u = src[p - s0], c = src[p];
+    for (int64_t z = z_start; z < z_end; ++z, p += s0) {
+      const T d = src[p + s0];
+      const T n = src[p - N2], s = src[p + N2], w = src[p - 1], e = src[p + 1];
+      if constexpr (KIND == K_STAR3D7) dst[p] = star3d7<T>(c, n, s, w, e, u, d, k);
+      else dst[p] = gradient3d<T>(c, n, s, w, e, u, d, k);
+      u = c;
+      c = d;
+    }
+  } else {
+    for (int64_t z = z_start; z < z_end; ++z) {
+      const int64_t p = z * s0 + y * N2 + x;
+      dst[p] = point_from_memory<T, KIND>(src, p, s0, N2, k);
+    }
   }
 }
 
@@ -133,13 +221,27 @@ __global__ void __launch_bounds__(256) naive_fdtd_kernel(T* __restrict__ ex, T* 
   }
 }
 
+template <typename T, int K>
+int wf_grid_t() {
+  static int grid = 0;
+  if (grid == 0) {
+    int dev = 0, sms = 0, per_sm = 0;
+    cudaGetDevice(&dev);
+    cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
+    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, generic_wf_kernel<T, K>, 256, 0);
+    grid = sms * (per_sm > 0 ? per_sm : 1);
+  }
+  return grid;
+}
+
 template <typename T>
 cudaError_t launch_generic_t(int kind, const GenericArgs& g, int grid, cudaStream_t s) {
   dim3 blk(256);
   switch (kind) {
 #define HEXS_CASE(K)                                                  \
   case K:                                                             \
-    generic_kernel<T, K><<<grid, blk, 0, s>>>(g);                     \
+    if (g.wf) generic_wf_kernel<T, K><<<wf_grid_t<T, K>(), blk, 0, s>>>(g); \
+    else generic_kernel<T, K><<<grid, blk, 0, s>>>(g);                \
     break;
     HEXS_CASE(K_JACOBI2D5) HEXS_CASE(K_STAR2D5) HEXS_CASE(K_BOX2D9) HEXS_CASE(K_FDTD2D)
     HEXS_CASE(K_STAR3D7) HEXS_CASE(K_GRADIENT3D) HEXS_CASE(K_BOX3D27) HEXS_CASE(K_GRADIENT2D)
@@ -172,11 +274,12 @@ cudaError_t launch_naive_t(int kind, int dims, const NaiveArgs& a, cudaStream_t 
       default: return cudaErrorInvalidValue;
     }
   } else {
-    dim3 grid((unsigned)((N2 - 2 + 255) / 256), (unsigned)(N1 - 2),
-              (unsigned)((N0 - 2 + kNaiveStrip - 1) / kNaiveStrip));
+    dim3 grid((unsigned)((N2 - 2 + 63) / 64), (unsigned)((N1 - 2 + 3) / 4),
+              (unsigned)((N0 - 2 + kNaive3DStrip - 1) / kNaive3DStrip));
+    dim3 blk(64, 4);
     switch (kind) {
 #define HEXS_CASE(K) \
-  case K: naive3d_kernel<T, K><<<grid, 256, 0, s>>>(src, dst, N0, N1, N2, k); break;
+  case K: naive3d_kernel<T, K><<<grid, blk, 0, s>>>(src, dst, N0, N1, N2, k); break;
       HEXS_CASE(K_STAR3D7) HEXS_CASE(K_GRADIENT3D) HEXS_CASE(K_BOX3D27)
 #undef HEXS_CASE
       default: return cudaErrorInvalidValue;
@@ -189,6 +292,11 @@ cudaError_t launch_naive_t(int kind, int dims, const NaiveArgs& a, cudaStream_t 
 
 cudaError_t launch_generic(int kind, int dtype, const GenericArgs& g, int grid, cudaStream_t s) {
   return dtype == 1 ? launch_generic_t<double>(kind, g, grid, s) : launch_generic_t<float>(kind, g, grid, s);
+}
+
+int generic_wf_grid(int kind, int dtype) {
+  (void)kind;
+  return dtype == 1 ? wf_grid_t<double, K_STAR3D7>() : wf_grid_t<float, K_STAR3D7>();
 }
 
 cudaError_t launch_naive(int kind, int dtype, int dims, const NaiveArgs& a, cudaStream_t s) {

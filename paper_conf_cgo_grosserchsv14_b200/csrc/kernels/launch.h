@@ -22,8 +22,17 @@ struct GenericArgs {
   int64_t Slo[2], Shi[2];
   double k0, k1;
   int32_t lo[kMaxH], hi[kMaxH];
+  // Wavefront execution of the classical tiles (wf = 1): persistent CTAs pull work items
+  // (S0, S1, S2) in anti-diagonal order of (S1, S2); a tile starts once its predecessors
+  // (S1-1, S2) and (S1, S2-1) of the same hexagon have published their completion flag.
+  int wf;
+  int64_t S0_hi;
+  int* flags;                   // [nS0][n1][n2], zeroed before the launch
+  unsigned long long* counter;  // work counter, zeroed before the launch
 };
 cudaError_t launch_generic(int kind, int dtype, const GenericArgs& g, int grid, cudaStream_t s);
+// Persistent grid size of the wavefront kernel (all CTAs co-resident).
+int generic_wf_grid(int kind, int dtype);
 
 // Naive one-step kernels (non-time-tiled comparator, K11).
 struct NaiveArgs {

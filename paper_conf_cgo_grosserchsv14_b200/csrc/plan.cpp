@@ -231,7 +231,8 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
       fast3d_tile(p->variant, &wy, &wx);
       wq = q == 0 ? wy : wx;
     } else if (wq <= 0) {
-      wq = (q == p->ncls - 1) ? 128 : 4;
+      if (d.dims == 3) wq = (q == p->ncls - 1) ? 64 : 8;  // wavefront tiles (y 8 x 64)
+      else wq = (q == p->ncls - 1) ? 128 : 4;
     }
     if (wq < 1) return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_plan: classical width must be >= 1");
     p->w[q] = wq;
@@ -286,6 +287,19 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
   // workspace: the second ping-pong buffer, 256-B granular
   p->ws_bytes = 0;
   if (d.pingpong && T_steps > 0) p->ws_bytes = ((size_t)d.points() * d.elem() + 255) / 256 * 256;
+  // 3D generic executor: classical tiles run as a dependence wavefront; per-tile completion
+  // flags and a work counter follow the ping-pong buffer in the workspace.
+  p->wavefront = (ex == EXEC_GENERIC && d.dims == 3 && p->ncls == 2);
+  if (p->wavefront && !p->launches.empty()) {
+    int64_t max_items = 0;
+    for (const Launch& l : p->launches)
+      max_items = std::max<int64_t>(max_items, (l.S0_hi - l.S0_lo + 1) * (l.Shi[0] - l.Slo[0] + 1) *
+                                                   (l.Shi[1] - l.Slo[1] + 1));
+    p->flag_off = p->ws_bytes;
+    p->flag_bytes = ((size_t)max_items * sizeof(int) + 255) / 256 * 256;
+    p->counter_off = p->flag_off + p->flag_bytes;
+    p->ws_bytes = p->counter_off + 256;
+  }
   *out = guard.release();
   return STENCIL_OK;
 }

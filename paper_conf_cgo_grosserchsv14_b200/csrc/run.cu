@@ -178,6 +178,14 @@ stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* 
           for (int f = 0; f < 3; ++f) g.f[f] = out[f];
         }
         fill_generic(p, l, g);
+        g.S0_hi = l.S0_hi;
+        if (p.wavefront) {
+          char* ws = static_cast<char*>(p.ws);
+          g.wf = 1;
+          g.flags = reinterpret_cast<int*>(ws + p.flag_off);
+          g.counter = reinterpret_cast<unsigned long long*>(ws + p.counter_off);
+          HEXS_CUDA(cudaMemsetAsync(ws + p.flag_off, 0, p.flag_bytes + 256, s), "stencil_run: reset tile flags");
+        }
         HEXS_CUDA(launch_generic(d.kind, d.dtype, g, grid, s), "stencil_run: generic kernel launch");
       }
       ev_end(s);
