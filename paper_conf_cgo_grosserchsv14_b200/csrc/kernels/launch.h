@@ -70,16 +70,21 @@ struct FdtdArgs {
 cudaError_t launch_fdtd(int variant, const FdtdArgs& a, int grid, cudaStream_t s);
 
 // 3D fast kernel.
+// 3D fast kernel (wavefront of smem-resident classical tiles, kernels/hex3d.cu).
 struct Fast3DArgs {
   void* buf[2];
   int64_t N0, N1, N2;
   int64_t tau0;
   int a_lo, a_hi, a_final;
-  int64_t S0_lo, row_off;
-  int W;
+  int64_t S0_lo, S0_hi, row_off;
+  int W, H, L, Q;          // box width, h, levels 2h+2, buffer planes (max rows + 2)
+  int64_t S1_lo, n1, S2_lo, n2;
   double k0, k1;
-  void* scratch;  // carry scratch (if any)
+  int* flags;
+  unsigned long long* counter;
+  int32_t lo[kMaxH], hi[kMaxH];
 };
 cudaError_t launch_fast3d(int variant, const Fast3DArgs& a, int grid, cudaStream_t s);
+constexpr int kFast3DNY = 16, kFast3DNX = 32;  // classical tile of the 3D fast kernel
 
 }  // namespace hexs

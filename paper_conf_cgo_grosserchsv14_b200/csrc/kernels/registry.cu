@@ -41,8 +41,19 @@ cudaError_t launch_fast2d(int variant, const Fast2DArgs& a, int grid, cudaStream
 // Not yet specialised: FDTD-2D and 3D classes run the generic hybrid kernel.
 int fdtd_variant(int, int, int) { return -1; }
 cudaError_t launch_fdtd(int, const FdtdArgs&, int, cudaStream_t) { return cudaErrorInvalidValue; }
-int fast3d_variant(int, int, int, int) { return -1; }
-int fast3d_tile(int, int* wy, int* wx) { *wy = 0; *wx = 0; return -1; }
-cudaError_t launch_fast3d(int, const Fast3DArgs&, int, cudaStream_t) { return cudaErrorInvalidValue; }
+// 3D fast kernel: any (h, w0) whose two level buffers fit in shared memory
+// (2 * (w0 + 2h + 3) planes x 18 lines x 40 columns).
+int fast3d_variant(int kind, int dtype, int h, int w0) {
+  if (kind != K_STAR3D7 && kind != K_GRADIENT3D && kind != K_BOX3D27) return -1;
+  const int Q = w0 + 2 * h + 3;
+  const size_t smem = (size_t)2 * Q * (kFast3DNY + 2) * (kFast3DNX + 8) * (dtype == 1 ? 8 : 4);
+  if (smem > 200 * 1024 || 2 * h + 2 > kMaxH) return -1;
+  return kind * 2 + dtype;
+}
+int fast3d_tile(int, int* wy, int* wx) {
+  *wy = kFast3DNY;
+  *wx = kFast3DNX;
+  return 0;
+}
 
 }  // namespace hexs

@@ -289,7 +289,7 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
   if (d.pingpong && T_steps > 0) p->ws_bytes = ((size_t)d.points() * d.elem() + 255) / 256 * 256;
   // 3D generic executor: classical tiles run as a dependence wavefront; per-tile completion
   // flags and a work counter follow the ping-pong buffer in the workspace.
-  p->wavefront = (ex == EXEC_GENERIC && d.dims == 3 && p->ncls == 2);
+  p->wavefront = ((ex == EXEC_GENERIC || ex == EXEC_FAST3D) && d.dims == 3 && p->ncls == 2);
   if (p->wavefront && !p->launches.empty()) {
     int64_t max_items = 0;
     for (const Launch& l : p->launches)

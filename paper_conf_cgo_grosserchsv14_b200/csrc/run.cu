@@ -164,10 +164,26 @@ stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* 
         a.a_hi = l.a_hi;
         a.a_final = a_final;
         a.S0_lo = l.S0_lo;
+        a.S0_hi = l.S0_hi;
         a.row_off = l.row_off;
         a.W = p.W;
+        a.H = p.h;
+        a.L = p.H;
+        a.Q = p.w0 + 2 * p.h + 3;
+        a.S1_lo = l.Slo[0];
+        a.n1 = l.Shi[0] - l.Slo[0] + 1;
+        a.S2_lo = l.Slo[1];
+        a.n2 = l.Shi[1] - l.Slo[1] + 1;
         a.k0 = d.coef[0];
         a.k1 = d.coef[1];
+        for (int q = 0; q < p.H; ++q) {
+          a.lo[q] = p.lo[q];
+          a.hi[q] = p.hi[q];
+        }
+        char* ws = static_cast<char*>(p.ws);
+        a.flags = reinterpret_cast<int*>(ws + p.flag_off);
+        a.counter = reinterpret_cast<unsigned long long*>(ws + p.counter_off);
+        HEXS_CUDA(cudaMemsetAsync(ws + p.flag_off, 0, p.flag_bytes + 256, s), "stencil_run: reset tile flags");
         HEXS_CUDA(launch_fast3d(p.variant, a, grid, s), "stencil_run: fast3d kernel launch");
       } else {
         GenericArgs g{};
