@@ -114,20 +114,34 @@ struct Tile {
   __device__ __forceinline__ int lo(int a) const { return g.lo[a]; }
   __device__ __forceinline__ int hi(int a) const { return g.hi[a]; }
 
-  // Issue the loads that complete the input buffer of level a: every input plane in full
-  // if `all`, else the In planes in full and the carry lines/columns of the planes computed
-  // at level a-1.
-  __device__ __forceinline__ void prefetch(int a, bool all) const {
+  // The In planes of level a (planes not computed at level a-1; every input plane if
+  // `all`) in full, into the input buffer of level a.  No dependence inside the launch:
+  // they were produced by earlier launches.
+  __device__ __forceinline__ void fetch_in_planes(int a, bool all) const {
     const int which = a & 1;
-    const int qlo = lo(a), qhi = hi(a) + 2;  // input planes q = b + 1, b in [lo-1, hi+1]
-    for (int q = qlo; q <= qhi; ++q) {
+    for (int q = lo(a); q <= hi(a) + 2; ++q) {
       const int b = q - 1;
-      const bool computed = !all && b >= lo(a - 1) && b <= hi(a - 1);
-      if (!computed) {
-        fetch(a, which, q, 0, LY, 0, NX + 2);
-      } else {
-        fetch(a, which, q, 0, 2, 0, NX + 2);   // carry lines (tile above, corner)
-        fetch(a, which, q, 2, LY, 0, 2);       // carry columns (tile to the left)
+      if (all || b < lo(a - 1) || b > hi(a - 1)) fetch(a, which, q, 0, LY, 0, NX + 2);
+    }
+  }
+  // The carries of level a: for every plane computed at level a-1, the two lines above the
+  // window (from tiles (S1-1, S2) and (S1-1, S2-1)) and the two columns left of it (from
+  // (S1, S2-1)), produced by those tiles at level a-1 in this launch.
+  __device__ __forceinline__ void fetch_carries(int a) const {
+    const int which = a & 1;
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    const T* src = static_cast<const T*>(g.buf[(g.tau0 + a) & 1]);
+    for (int q = lo(a - 1) + 1; q <= hi(a - 1) + 1; ++q) {
+      fetch(a, which, q, 0, 2, 0, NX + 2);
+      // two columns x NY lines: one pass of one warp (lane = 2 * line + column)
+      if (warp == (q & 3)) {
+        const int ly = 2 + (lane >> 1), lx = lane & 1;
+        int64_t z, y, x;
+        pos(a - 1, q, ly, lx, z, y, x);
+        z = z < 0 ? 0 : (z >= g.N0 ? g.N0 - 1 : z);
+        y = y < 0 ? 0 : (y >= g.N1 ? g.N1 - 1 : y);
+        x = x < 0 ? 0 : (x >= g.N2 ? g.N2 - 1 : x);
+        cp_async(bufp(which, q, ly, lx), src + z * plane + y * g.N2 + x);
       }
     }
   }
@@ -164,12 +178,6 @@ __global__ void __launch_bounds__(NT, 3) fast3d_kernel(const __grid_constant__ A
           }
           off += pairs * ns0;
         }
-        const int64_t base = (S0 - g.S0_lo) * n1 * n2;
-        if (q1 > 0)
-          while (ld_acquire(g.flags + base + (q1 - 1) * n2 + q2) == 0) __nanosleep(32);
-        if (q2 > 0)
-          while (ld_acquire(g.flags + base + q1 * n2 + q2 - 1) == 0) __nanosleep(32);
-        __threadfence();
       }
       item_s[0] = S0;
       item_s[1] = q1;
@@ -178,18 +186,38 @@ __global__ void __launch_bounds__(NT, 3) fast3d_kernel(const __grid_constant__ A
     __syncthreads();
     const int64_t S0 = item_s[0];
     if (S0 < 0) break;
-    Tile<T> t{g, sm, S0 * g.W - g.row_off, (g.S1_lo + item_s[1]) * NY, (g.S2_lo + item_s[2]) * NX, plane};
+    const int64_t q1 = item_s[1], q2 = item_s[2];
+    const int64_t fbase = (S0 - g.S0_lo) * n1 * n2;
+    int* my_flag = g.flags + fbase + q1 * n2 + q2;
+    Tile<T> t{g, sm, S0 * g.W - g.row_off, (g.S1_lo + q1) * NY, (g.S2_lo + q2) * NX, plane};
 
-    // prologue: the full input of the first level
-    t.prefetch(g.a_lo, true);
+    // prologue: every input plane of the first level (all produced by earlier launches)
+    t.fetch_in_planes(g.a_lo, true);
     cp_async_commit_wait();
     __syncthreads();
 
     for (int a = g.a_lo; a <= g.a_hi; ++a) {
       const int ib = a & 1, ob = (a + 1) & 1;
-      // (1) one level ahead: In planes + carries of level a+1 into the output buffer's
-      //     areas that level a does not write
-      if (a < g.a_hi) t.prefetch(a + 1, false);
+      if (a > g.a_lo) {
+        // (0) level-granular dependences: the predecessors (S1-1, S2), (S1, S2-1),
+        //     (S1-1, S2-1) must have published level a-1 (progress >= a - a_lo)
+        if (tid == 0) {
+          const int need = a - g.a_lo;
+          if (q1 > 0)
+            while (ld_acquire(g.flags + fbase + (q1 - 1) * n2 + q2) < need) __nanosleep(20);
+          if (q2 > 0)
+            while (ld_acquire(g.flags + fbase + q1 * n2 + q2 - 1) < need) __nanosleep(20);
+          if (q1 > 0 && q2 > 0)
+            while (ld_acquire(g.flags + fbase + (q1 - 1) * n2 + q2 - 1) < need) __nanosleep(20);
+          __threadfence();
+        }
+        __syncthreads();
+        t.fetch_carries(a);
+        cp_async_commit_wait();  // also completes the In planes prefetched during level a-1
+        __syncthreads();
+      }
+      // (1) one level ahead: the In planes of level a+1 into areas level a does not write
+      if (a < g.a_hi) t.fetch_in_planes(a + 1, false);
       // (2) compute level a: rows [lo, hi] split in two groups, 3-plane register window
       const int rlo = t.lo(a), rhi = t.hi(a);
       const int mid = (rlo + rhi) >> 1;
@@ -270,7 +298,6 @@ __global__ void __launch_bounds__(NT, 3) fast3d_kernel(const __grid_constant__ A
             }
         }
       }
-      cp_async_commit_wait();
       __syncthreads();
       // (3) copy out: Out planes / final level in full, else the successors' carries
       T* dst = static_cast<T*>(g.buf[(g.tau0 + a + 1) & 1]);
@@ -303,13 +330,13 @@ __global__ void __launch_bounds__(NT, 3) fast3d_kernel(const __grid_constant__ A
             dst[zz * plane + y * g.N2 + x] = *t.bufp(ob, r + 1, ly, lx);
         }
       }
-      // no barrier: the next level writes buffer a&1, the copy-out above reads (a+1)&1
+      __syncthreads();  // every thread's stores of level a precede the release
+      if (tid == 0) {
+        __threadfence();
+        st_release(my_flag, a - g.a_lo + 1);
+      }
     }
-    __syncthreads();  // every thread's stores of this tile precede the release
-    if (tid == 0) {
-      __threadfence();
-      st_release(g.flags + (S0 - g.S0_lo) * n1 * n2 + item_s[1] * n2 + item_s[2], 1);
-    }
+    cp_async_commit_wait();
   }
 }
 
