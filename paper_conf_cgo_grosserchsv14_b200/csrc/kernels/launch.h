@@ -86,5 +86,6 @@ struct Fast3DArgs {
 };
 cudaError_t launch_fast3d(int variant, const Fast3DArgs& a, int grid, cudaStream_t s);
 constexpr int kFast3DNY = 16, kFast3DNX = 32;  // classical tile of the 3D fast kernel
+size_t fast3d_smem_bytes(int dtype, int Q);
 
 }  // namespace hexs

@@ -46,8 +46,7 @@ cudaError_t launch_fdtd(int, const FdtdArgs&, int, cudaStream_t) { return cudaEr
 int fast3d_variant(int kind, int dtype, int h, int w0) {
   if (kind != K_STAR3D7 && kind != K_GRADIENT3D && kind != K_BOX3D27) return -1;
   const int Q = w0 + 2 * h + 3;
-  const size_t smem = (size_t)2 * Q * (kFast3DNY + 2) * (kFast3DNX + 8) * (dtype == 1 ? 8 : 4);
-  if (smem > 200 * 1024 || 2 * h + 2 > kMaxH) return -1;
+  if (fast3d_smem_bytes(dtype, Q) > 200 * 1024 || 2 * h + 2 > kMaxH) return -1;
   return kind * 2 + dtype;
 }
 int fast3d_tile(int, int* wy, int* wx) {

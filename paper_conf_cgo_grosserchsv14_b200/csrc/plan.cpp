@@ -215,7 +215,8 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
         ex = EXEC_FAST2D;
     } else {
       p->variant = fast3d_variant(d.kind, dtype, h, w0);
-      if (p->variant >= 0 && p->hd == 0) ex = EXEC_FAST3D;
+      // TMA tensor maps need 16-B aligned plane/line strides (N2 * elem % 16 == 0)
+      if (p->variant >= 0 && p->hd == 0 && (d.ext[2] * (int64_t)d.elem()) % 16 == 0) ex = EXEC_FAST3D;
     }
   } else if (flags != STENCIL_EXEC_GENERIC) {
     return fail(STENCIL_E_INVALID, "stencil_plan: unknown tile.flags");

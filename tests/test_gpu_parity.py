@@ -121,10 +121,21 @@ def test_fdtd_tiles(h, w0):
 @pytest.mark.parametrize("dtype", [np.float32, np.float64])
 @pytest.mark.parametrize("executor", ["auto", "generic", "naive"])
 def test_3d(kind, dtype, executor):
-    for shape, T in [((34, 29, 67), 7), ((20, 40, 33), 12)]:
+    # unaligned rows run the generic wavefront; rows with 16-B aligned strides the TMA kernel
+    for shape, T in [((34, 29, 67), 7), ((20, 40, 33), 12), ((30, 37, 68), 9), ((23, 51, 100), 13)]:
         g = stencil_inputs.uniform(shape, seed=30, dtype=dtype)
-        got, _ = _gpu_run(kind, g, T, dtype, executor=executor)
+        got, plan = _gpu_run(kind, g, T, dtype, executor=executor)
+        if executor == "auto" and shape[2] % 4 == 0:
+            assert plan.info["fast_kernel"] == 1
         assert_bitexact(got, oracle.run(kind, g, T), f"{kind} {executor} {shape}")
+
+
+@pytest.mark.parametrize("h,w0", [(2, 7), (1, 3), (3, 2)])
+def test_fast3d_tiles(h, w0):
+    g = stencil_inputs.uniform((41, 70, 96), seed=31)
+    got, plan = _gpu_run("star3d7", g, 11, np.float32, h=h, w0=w0)
+    assert plan.info["fast_kernel"] == 1
+    assert_bitexact(got, oracle.run("star3d7", g, 11), f"fast3d h={h} w0={w0}")
 
 
 def test_constant_field_full_size_property():
