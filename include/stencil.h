@@ -143,6 +143,7 @@ typedef struct {
   int32_t hex_dim;
   int32_t delta0_num, delta0_den, delta1_num, delta1_den; /* cone slopes along hex_dim */
   int32_t delta_cls[3];  /* classical skews delta1_i for the other dims (slow -> fast) */
+  int32_t trans_cls[3];  /* classical tile translation offsets (Sec. 4.2.3) */
   int32_t h, w0, w[3];   /* effective tile parameters */
   int32_t H, W;          /* box height 2h+2 and width 2w0+2+floor(d0 h)+floor(d1 h) */
   int32_t F0, F1;        /* floor(delta0 h), floor(delta1 h) */
@@ -178,7 +179,8 @@ stencil_status stencil_plan_launches(stencil_plan_t plan, stencil_launch_t *out,
 stencil_status stencil_plan_hexagon(stencil_plan_t plan, int32_t *lo, int32_t *hi, int32_t cap);
 
 /* Schedule of one instance (canonical time tau, spatial point s[dims]) as the tuple
- * [T, p, S0, S_1..S_n, t', s'_0, s'_1..s'_n] of Sec. 3.6 (n = dims-1 classical dims in
+ * [T, p, S0, S_1..S_n, t', s'_0, s'_1..s'_n] of Sec. 3.6 (eq. (14) with the plan's classical skews
+ * and translation offsets; n = dims-1 classical dims in
  * slow -> fast order excluding hex_dim), written to sched (capacity 2*dims+3). */
 stencil_status stencil_plan_schedule_of(stencil_plan_t plan, int64_t tau, const int64_t *s,
                                         int64_t *sched);

@@ -227,16 +227,19 @@ def hex_tile(hx: Hex, t: int, s0: int, literal_eq3: bool = False):
     return out
 
 
-def classical(delta1_i: Fr, w_i: int, s_i: int, u: int) -> Tuple[int, int]:
+def classical(delta1_i: Fr, w_i: int, s_i: int, u: int, trans: int = 0) -> Tuple[int, int]:
     """Eq. (14) S_i = floor((s_i + delta1_i u)/w_i) and eq. (17)
     s'_i = (s_i + delta1_i u) mod w_i, with u the per-phase normalised time of eqs. (15),
-    (16) (PAPER.md:559-591)."""
-    x = s_i + delta1_i * u
+    (16); `trans` translates the tiles by a fixed offset ("We allow the
+    tiles in the schedule to be translated by manually specifying the translation offset",
+    Sec. 4.2.3, PAPER.md:761-763)."""
+    x = s_i - trans + delta1_i * u
     S = floor(x / w_i)
     return S, x - S * w_i
 
 
-def hybrid(hx: Hex, deltas_i: Sequence[Fr], w: Sequence[int], t: int, s: Sequence[int]):
+def hybrid(hx: Hex, deltas_i: Sequence[Fr], w: Sequence[int], t: int, s: Sequence[int],
+           trans: Sequence[int] = None):
     """[t, s0..sn] -> [T, p, S0..Sn, t', s'0..s'n] (Sec. 3.6, PAPER.md:596-603).  The
     normalised u of eqs. (15)/(16) equals the local box row a."""
     tiles = hex_tile(hx, t, s[0])
@@ -244,7 +247,7 @@ def hybrid(hx: Hex, deltas_i: Sequence[Fr], w: Sequence[int], t: int, s: Sequenc
     T, p, S0, a, b = tiles[0]
     Ss, sp = [], []
     for i in range(1, len(s)):
-        Si, si = classical(deltas_i[i - 1], w[i - 1], s[i], a)
+        Si, si = classical(deltas_i[i - 1], w[i - 1], s[i], a, trans[i - 1] if trans else 0)
         Ss.append(Si)
         sp.append(si)
     return (T, p, S0, *Ss, a, b, *sp)
@@ -277,7 +280,8 @@ def hexagon_rows(hx: Hex) -> List[Tuple[int, int]]:
 
 
 def check_schedule(prog: Program, N: Sequence[int], steps: int, hx: Hex,
-                   deltas_i: Sequence[Fr], w: Sequence[int], literal_eq3: bool = False):
+                   deltas_i: Sequence[Fr], w: Sequence[int], literal_eq3: bool = False,
+                   trans: Sequence[int] = None):
     """Brute-force validity of the hybrid schedule on a small grid: returns a dict of
     violation counts (all zero for a valid schedule)."""
     sched = {}
@@ -288,7 +292,8 @@ def check_schedule(prog: Program, N: Sequence[int], steps: int, hx: Hex,
             coverage_err += 1
             continue
         T, p, S0, a, b = tiles[0]
-        Ss = [classical(deltas_i[i - 1], w[i - 1], s[i], a)[0] for i in range(1, len(s))]
+        Ss = [classical(deltas_i[i - 1], w[i - 1], s[i], a, trans[i - 1] if trans else 0)[0]
+              for i in range(1, len(s))]
         sched[(tau, s)] = ((T, p), S0, tuple(Ss) + (a,))
     order_err = same_phase_err = same_step_err = 0
     for src, snk in dependences(prog, N, steps):

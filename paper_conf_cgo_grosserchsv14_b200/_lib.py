@@ -44,7 +44,7 @@ class PlanInfo(ctypes.Structure):
                 ("hex_dim", ctypes.c_int32),
                 ("delta0_num", ctypes.c_int32), ("delta0_den", ctypes.c_int32),
                 ("delta1_num", ctypes.c_int32), ("delta1_den", ctypes.c_int32),
-                ("delta_cls", ctypes.c_int32 * 3), ("h", ctypes.c_int32), ("w0", ctypes.c_int32),
+                ("delta_cls", ctypes.c_int32 * 3), ("trans_cls", ctypes.c_int32 * 3), ("h", ctypes.c_int32), ("w0", ctypes.c_int32),
                 ("w", ctypes.c_int32 * 3), ("H", ctypes.c_int32), ("W", ctypes.c_int32),
                 ("F0", ctypes.c_int32), ("F1", ctypes.c_int32), ("executor", ctypes.c_int32),
                 ("fast_kernel", ctypes.c_int32), ("n_launches", ctypes.c_int64),

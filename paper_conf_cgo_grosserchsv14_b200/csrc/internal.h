@@ -76,6 +76,7 @@ struct Plan {
   int cls[2] = {0, 0};  // classical dims (slow -> fast)
   Rat d0, d1;           // cone slopes along hd
   int dcls[2] = {0, 0}; // integer classical skews delta1_i
+  int ctrans[2] = {0, 0};  // classical tile translation offsets (Sec. 4.2.3)
   int h = 0, w0 = 0, w[2] = {1, 1};
   int H = 0, W = 0, F0 = 0, F1 = 0, c = 0;
   std::vector<int32_t> lo, hi;  // hexagon rows per level a

@@ -4,25 +4,27 @@
 //
 // Mapping:
 //   * work item = one classical tile (S1, S2) of one hexagon S0 of the launch's (T, p): a
-//     NY x NX (y, x) parallelogram over the hexagon's 2h+2 levels and rows z;
+//     NY x NX (y, x) parallelogram over the hexagon's 2h+2 levels and rows z.  Skews: y by 1
+//     per level (delta1_y = 1), x by 4 per level with a +1 tile translation (Sec. 4.2.3,
+//     PAPER.md:755-763) so that every x-window this kernel moves starts on a 16-B boundary
+//     (the TMA unit requires it; any skew >= delta1_x keeps eq. (14) valid -- reading R16);
 //   * items run as a dependence WAVEFRONT at LEVEL granularity: level a of (S1, S2) needs
-//     level a-1 of (S1-1, S2), (S1, S2-1), (S1-1, S2-1) (the skew of eq. (14) makes every
-//     dependence point to a lower tile index).  Persistent CTAs fetch items in anti-diagonal
-//     order from an atomic counter; progress flags (levels done) are published with
-//     st.release after the tile's carries are in global memory.  So the ~26-51 hexagons per
-//     phase of a 512^3 grid keep all 148 SMs busy -- the paper's mapping runs S1..Sn
+//     level a-1 of (S1-1, S2), (S1, S2-1), (S1-1, S2-1).  Persistent CTAs fetch items in
+//     anti-diagonal order from an atomic counter; progress flags (levels done) are published
+//     with st.release after the tile's carries are in global memory, so the ~26-51 hexagons
+//     per phase of a 512^3 grid keep all 148 SMs busy -- the paper's mapping runs S1..Sn
 //     sequentially inside one block;
 //   * the tile's current level lives in shared memory (two level buffers: planes z x 18
-//     lines x 36 columns); a thread owns 2 lines x 4 columns of one half of the rows and
+//     lines x 40 columns); a thread owns 2 lines x 4 columns of one half of the rows and
 //     sweeps z with a 3-plane register window (z-neighbours from registers, y/x neighbours
 //     from LDS.128 + LDS.64);
 //   * everything a tile reads from L2/HBM arrives by 3-D TMA tensor copies
 //     (cp.async.bulk.tensor.3d, SASS UTMALDG) completing on one mbarrier per level buffer:
 //     the In planes of level a+1 (the hexagon's slanted-edge inputs) one
-//     level ahead, the carries (2 lines above / 2 columns left, produced by the predecessor
+//     level ahead, the carries (2 lines above / 5 columns left, produced by the predecessor
 //     tiles in this launch) when their flags allow; out-of-grid box elements are zero-filled
 //     by the TMA unit and never used;
-//   * results leave from registers: the Out planes, the tile's last two lines and columns
+//   * results leave from registers: the Out planes, the tile's last 2 lines and 5 columns
 //     (its successors' carries) and the final level -- interleaved copy-out.
 #include <cuda.h>
 #include <cudaTypedefs.h>
@@ -38,9 +40,11 @@ namespace fast3d {
 
 constexpr int NY = kFast3DNY, NX = kFast3DNX;  // classical tile (y lines, x columns)
 constexpr int NT = 128;                        // 2 row groups x 8 line pairs x 8 column quads
+constexpr int SIGMA = 4;                       // x skew per level
+constexpr int CL = SIGMA + 1;                  // left carry columns (skew + stencil radius)
 constexpr int LY = NY + 2;                     // buffer lines: 2 carry lines + NY
-constexpr int SX = NX + 4;                     // buffer columns: 2 carry + NX + 2 (TMA box width)
-constexpr int CW = 4;                          // carry-column box width (16 B of fp32)
+constexpr int SX = 40;                         // buffer columns: CL carry + NX window (+3), TMA box
+constexpr int CW = 8;                          // carry-column box width (two 16-B groups of fp32)
 // plane pitch (elements), padded so every TMA destination is 128-B aligned
 template <typename T> constexpr int PP = ((LY * SX * (int)sizeof(T) + 127) / 128 * 128) / (int)sizeof(T);
 template <typename T> constexpr size_t smem_bytes(int Q) {
@@ -88,6 +92,13 @@ __device__ __forceinline__ T apply(const T (&x)[3][3][3], const Coef<T>& k) {
   }
 }
 
+// Buffer conventions.  The input buffer of level a (level a-1 values) has its column 0 at
+// x = X0 - 4a (16-B aligned) and its line 0 at y = Y0 - a - 1: columns [0, CL) and lines
+// {0, 1} are carries, the tile's own level-(a-1) window sits at columns [CL, CL + NX) and
+// lines [2, LY).  Level a's output window (x in [X0-4a+1, X0-4a+NX], y in [Y0-a, Y0-a+NY))
+// is written into the other buffer in ITS convention (column = x - (X0 - 4(a+1)),
+// line = y - (Y0 - a - 2)).  A thread (lp, xq) computes outputs x = X0-4a+1+4xq+j,
+// y = Y0-a+2lp+i, whose inputs sit at input columns [4xq, 4xq+5] and lines [2lp, 2lp+3].
 template <typename T, int KIND>
 __global__ void __launch_bounds__(NT, 2) fast3d_kernel(const __grid_constant__ Fast3DArgs g,
                                                        const __grid_constant__ Maps m) {
@@ -95,8 +106,7 @@ __global__ void __launch_bounds__(NT, 2) fast3d_kernel(const __grid_constant__ F
   __shared__ __align__(8) uint64_t mbar[2];
   __shared__ int64_t item_s[3];
   T* buf = reinterpret_cast<T*>((reinterpret_cast<uintptr_t>(smem_raw) + 127) & ~uintptr_t(127));
-  // buf: [2][Q] planes of PP elements ([LY][SX] used); side: [Q][NY][CW]
-  T* side = buf + (size_t)2 * g.Q * PP<T>;
+  T* side = buf + (size_t)2 * g.Q * PP<T>;  // [Q][NY][CW] landing area of the carry columns
   auto B = [&](int which, int q, int ly, int lx) -> T* {
     return buf + ((size_t)which * g.Q + q) * PP<T> + ly * SX + lx;
   };
@@ -158,7 +168,7 @@ __global__ void __launch_bounds__(NT, 2) fast3d_kernel(const __grid_constant__ F
         mbar_arrive_expect_tx(&mbar[ib], plane_bytes * (qhi - qlo + 1));
         const CUtensorMap* mp = &m.plane[(g.tau0 + a) & 1];
         for (int q = qlo; q <= qhi; ++q)
-          tma_3d(B(ib, q, 0, 0), mp, (int)(X0 - a - 1), (int)(Y0 - a - 1), (int)(i0 + q - 1), &mbar[ib]);
+          tma_3d(B(ib, q, 0, 0), mp, (int)(X0 - SIGMA * a), (int)(Y0 - a - 1), (int)(i0 + q - 1), &mbar[ib]);
       }
       mbar_wait_parity(&mbar[ib], phase[ib]);
       phase[ib] ^= 1u;
@@ -180,18 +190,19 @@ __global__ void __launch_bounds__(NT, 2) fast3d_kernel(const __grid_constant__ F
           fence_proxy_async_smem();
           mbar_arrive_expect_tx(&mbar[ib], (cline_bytes + ccol_bytes) * (phi - plo + 1));
           const int par = (int)((g.tau0 + a) & 1);
+          const int xo = (int)(X0 - SIGMA * a);
           for (int q = plo + 1; q <= phi + 1; ++q) {
             const int z = (int)(i0 + q - 1);
-            tma_3d(B(ib, q, 0, 0), &m.cline[par], (int)(X0 - a - 1), (int)(Y0 - a - 1), z, &mbar[ib]);
-            tma_3d(side + (size_t)q * NY * CW, &m.ccol[par], (int)(X0 - a - 1), (int)(Y0 - a + 1), z, &mbar[ib]);
+            tma_3d(B(ib, q, 0, 0), &m.cline[par], xo, (int)(Y0 - a - 1), z, &mbar[ib]);
+            tma_3d(side + (size_t)q * NY * CW, &m.ccol[par], xo, (int)(Y0 - a + 1), z, &mbar[ib]);
           }
         }
         mbar_wait_parity(&mbar[ib], phase[ib]);  // carries + the In planes issued at level a-1
         phase[ib] ^= 1u;
-        // the two carry columns of each computed plane into place
+        // the CL carry columns of each computed plane into place
         const int nc = phi - plo + 1;
-        for (int e = tid; e < nc * NY * 2; e += NT) {
-          const int q = plo + 1 + e / (NY * 2), l = (e >> 1) % NY, c = e & 1;
+        for (int e = tid; e < nc * NY * CL; e += NT) {
+          const int q = plo + 1 + e / (NY * CL), r = e % (NY * CL), l = r / CL, c = r % CL;
           *B(ib, q, 2 + l, c) = side[((size_t)q * NY + l) * CW + c];
         }
         __syncthreads();
@@ -207,14 +218,14 @@ __global__ void __launch_bounds__(NT, 2) fast3d_kernel(const __grid_constant__ F
         const CUtensorMap* mp = &m.plane[(g.tau0 + a + 1) & 1];
         for (int q = qlo; q <= qhi; ++q)
           if (q - 1 < g.lo[a] || q - 1 > g.hi[a])
-            tma_3d(B(ob, q, 0, 0), mp, (int)(X0 - a - 2), (int)(Y0 - a - 2), (int)(i0 + q - 1), &mbar[ob]);
+            tma_3d(B(ob, q, 0, 0), mp, (int)(X0 - SIGMA * (a + 1)), (int)(Y0 - a - 2), (int)(i0 + q - 1), &mbar[ob]);
       }
 
       // (2) compute level a: rows [lo, hi] in two groups, z-window rotated without copies
       const int rlo = g.lo[a], rhi = g.hi[a];
       const int mid = (rlo + rhi) >> 1;
       const int r0 = zg == 0 ? rlo : mid + 1, r1 = zg == 0 ? mid : rhi;
-      const int64_t yb = Y0 - a + 2 * lp, xb = X0 - a + 4 * xq;  // global y, x of output (0, 0)
+      const int64_t yb = Y0 - a + 2 * lp, xb = X0 - SIGMA * a + 1 + 4 * xq;  // output (0, 0)
       bool lineok[2], colok[4];
 #pragma unroll
       for (int i = 0; i < 2; ++i) lineok[i] = (yb + i >= 1) && (yb + i <= g.N1 - 2);
@@ -260,19 +271,17 @@ __global__ void __launch_bounds__(NT, 2) fast3d_kernel(const __grid_constant__ F
             const T v = apply<T, KIND>(x, cf);
             out[i][j] = (zok && lineok[i] && colok[j]) ? v : x[1][1][1];
           }
+        // into the output buffer: columns CL + 4xq + j (one scalar, one pair, one scalar)
 #pragma unroll
         for (int i = 0; i < 2; ++i) {
-          T* p = B(ob, r + 1, 2 + 2 * lp + i, 2 + 4 * xq);
-          if constexpr (sizeof(T) == 4) {
-            reinterpret_cast<float2*>(p)[0] = make_float2(out[i][0], out[i][1]);
-            reinterpret_cast<float2*>(p)[1] = make_float2(out[i][2], out[i][3]);
-          } else {
-            reinterpret_cast<double2*>(p)[0] = make_double2(out[i][0], out[i][1]);
-            reinterpret_cast<double2*>(p)[1] = make_double2(out[i][2], out[i][3]);
-          }
+          T* p = B(ob, r + 1, 2 + 2 * lp + i, CL + 4 * xq);
+          p[0] = out[i][0];
+          if constexpr (sizeof(T) == 4) reinterpret_cast<float2*>(p + 1)[0] = make_float2(out[i][1], out[i][2]);
+          else { p[1] = out[i][1]; p[2] = out[i][2]; }
+          p[3] = out[i][3];
         }
         // copy-out from registers: Out planes / final level in full, else the successors'
-        // carries (the window's last two lines and last two columns)
+        // carries (the window's last 2 lines and last CL columns)
         bool full = fin;
         if (a == g.H) full = full || r == rlo || r == rhi;
         else if (a > g.H && a < g.L - 1) full = full || r <= rlo + 1 || r >= rhi - 1;
@@ -283,7 +292,7 @@ __global__ void __launch_bounds__(NT, 2) fast3d_kernel(const __grid_constant__ F
           for (int i = 0; i < 2; ++i)
 #pragma unroll
             for (int j = 0; j < 4; ++j)
-              if (lineok[i] && colok[j] && (full || lp == 7 || (xq == 7 && j >= 2)))
+              if (lineok[i] && colok[j] && (full || lp == 7 || 4 * xq + j >= NX - CL))
                 zp[(yb + i) * g.N2 + xb + j] = out[i][j];
         }
       };

@@ -114,7 +114,8 @@ bool schedule_of(const Plan& p, int64_t tau, const int64_t* s, int64_t* sched) {
     sched[k++] = S0;
     int64_t sp[2] = {0, 0};
     for (int q = 0; q < p.ncls; ++q) {
-      const int64_t x = s[p.cls[q]] + (int64_t)p.dcls[q] * a;  // eqs. (14), (17)
+      // eqs. (14), (17) with the tile translation offset of Sec. 4.2.3
+      const int64_t x = s[p.cls[q]] - p.ctrans[q] + (int64_t)p.dcls[q] * a;
       const int64_t Si = floor_div(x, p.w[q]);
       sched[k++] = Si;
       sp[q] = x - Si * p.w[q];
@@ -239,6 +240,16 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
     p->w[q] = wq;
   }
 
+  // The 3D fast kernel moves whole 16-B groups with TMA, whose innermost box origin must be
+  // 16-B aligned: it skews the contiguous dimension by 4 per level (any integer skew >=
+  // delta1_i keeps eq. (14) valid, reading R16) and translates the x tiles by +1 (the
+  // translation offset of Sec. 4.2.3) so the inputs of a thread's four
+  // outputs start on a 16-B boundary.
+  if (ex == EXEC_FAST3D) {
+    p->dcls[1] = std::max(p->dcls[1], 4);
+    p->ctrans[1] = 1;
+  }
+
   // a3: launch table.  Order (T, 0), (T, 1), T ascending.
   int64_t dlo[3], dhi[3];
   for (int q = 0; q < d.dims; ++q) {
@@ -276,8 +287,8 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
           ln.Slo[q] = ln.Shi[q] = 0;
           if (q < p->ncls) {
             const int dq = p->cls[q];
-            ln.Slo[q] = floor_div(dlo[dq] + (int64_t)p->dcls[q] * ln.a_lo, p->w[q]);
-            ln.Shi[q] = floor_div(dhi[dq] + (int64_t)p->dcls[q] * ln.a_hi, p->w[q]);
+            ln.Slo[q] = floor_div(dlo[dq] - p->ctrans[q] + (int64_t)p->dcls[q] * ln.a_lo, p->w[q]);
+            ln.Shi[q] = floor_div(dhi[dq] - p->ctrans[q] + (int64_t)p->dcls[q] * ln.a_hi, p->w[q]);
           }
         }
         p->launches.push_back(ln);
@@ -369,6 +380,7 @@ stencil_status stencil_plan_info(stencil_plan_t plan, stencil_plan_info_t* info)
   o.delta1_num = (int32_t)p->d1.n;
   o.delta1_den = (int32_t)p->d1.d;
   for (int q = 0; q < 3; ++q) o.delta_cls[q] = q < p->ncls ? p->dcls[q] : 0;
+  for (int q = 0; q < 3; ++q) o.trans_cls[q] = q < p->ncls ? p->ctrans[q] : 0;
   o.h = p->h;
   o.w0 = p->w0;
   for (int q = 0; q < 3; ++q) o.w[q] = q < p->ncls ? p->w[q] : 0;

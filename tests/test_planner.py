@@ -79,7 +79,8 @@ def _oracle_sched(kind, plan, tau, s):
                info["h"], info["w0"])
     dims = len(s)
     ncls = dims - 1
-    return S.hybrid(hx, [Fr(x) for x in info["delta_cls"][:ncls]], info["w"][:ncls], tau, s)
+    return S.hybrid(hx, [Fr(x) for x in info["delta_cls"][:ncls]], info["w"][:ncls], tau, s,
+                    info["trans_cls"][:ncls])
 
 
 @pytest.mark.parametrize("kind,N,T,h,w0,w", [

@@ -156,3 +156,15 @@ def test_fdtd_hybrid_schedule_valid(h, w0, w1):
     assert w0 >= S.w0_lower_bound(hx.d0, hx.d1, h)
     r = S.check_schedule(S.FDTD2D, (22, 11), 8, hx, [Fr(1)], [w1])
     assert r["coverage"] == r["order"] == r["same_phase"] == r["same_step"] == 0, r
+
+
+@pytest.mark.parametrize("offsets", [S.STAR3D7, S.BOX3D27])
+def test_larger_skew_and_translation_stay_valid(offsets):
+    """The 3D kernel skews x by 4 per level (>= delta1_x = 1) and translates x tiles by +1
+    (Sec. 4.2.3's translation offset): still exactly-once and
+    dependence-respecting (reading R16)."""
+    prog = S.single_statement(offsets)
+    N = (12, 7, 19)
+    r = S.check_schedule(prog, N, 7, S.Hex(Fr(1), Fr(1), 1, 1), [Fr(1), Fr(4)], [3, 8],
+                         trans=[0, 1])
+    assert r["coverage"] == r["order"] == r["same_phase"] == r["same_step"] == 0, r
