@@ -39,7 +39,9 @@ namespace hexs {
 namespace fast3d {
 
 constexpr int NY = kFast3DNY, NX = kFast3DNX;  // classical tile (y lines, x columns)
-constexpr int NT = 128;                        // 2 row groups x 8 line pairs x 8 column quads
+constexpr int NLP = NY / 2;                    // line pairs per tile
+constexpr int NT = 2 * NLP * 8;                // 2 row groups x NLP line pairs x 8 column quads
+constexpr int MINB = NY <= 8 ? 4 : 2;          // resident CTAs per SM (shared-memory bound)
 constexpr int SIGMA = 4;                       // x skew per level
 constexpr int CL = SIGMA + 1;                  // left carry columns (skew + stencil radius)
 constexpr int LY = NY + 2;                     // buffer lines: 2 carry lines + NY
@@ -65,6 +67,13 @@ __device__ __forceinline__ int ld_acquire(const int* p) {
 __device__ __forceinline__ void st_release(int* p, int v) {
   asm volatile("st.release.gpu.global.b32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
 }
+__device__ __forceinline__ long long gtimer() {
+  long long t;
+  asm volatile("mov.u64 %0, %globaltimer;" : "=l"(t));
+  return t;
+}
+constexpr int kTraceStride = 32;  // per item: [sm, start, prologue, (flag, data, done) per level]
+
 __device__ __forceinline__ void mbar_expect_tx(uint64_t* bar, uint32_t bytes) {
   asm volatile("mbarrier.expect_tx.relaxed.cta.shared::cta.b64 [%0], %1;" ::"r"(smem_u32(bar)), "r"(bytes)
                : "memory");
@@ -100,11 +109,12 @@ __device__ __forceinline__ T apply(const T (&x)[3][3][3], const Coef<T>& k) {
 // line = y - (Y0 - a - 2)).  A thread (lp, xq) computes outputs x = X0-4a+1+4xq+j,
 // y = Y0-a+2lp+i, whose inputs sit at input columns [4xq, 4xq+5] and lines [2lp, 2lp+3].
 template <typename T, int KIND>
-__global__ void __launch_bounds__(NT, 2) fast3d_kernel(const __grid_constant__ Fast3DArgs g,
+__global__ void __launch_bounds__(NT, MINB) fast3d_kernel(const __grid_constant__ Fast3DArgs g,
                                                        const __grid_constant__ Maps m) {
   extern __shared__ __align__(128) unsigned char smem_raw[];
   __shared__ __align__(8) uint64_t mbar[2];
   __shared__ int64_t item_s[3];
+  __shared__ int64_t trace_it_s;
   T* buf = reinterpret_cast<T*>((reinterpret_cast<uintptr_t>(smem_raw) + 127) & ~uintptr_t(127));
   T* side = buf + (size_t)2 * g.Q * PP<T>;  // [Q][NY][CW] landing area of the carry columns
   auto B = [&](int which, int q, int ly, int lx) -> T* {
@@ -112,7 +122,7 @@ __global__ void __launch_bounds__(NT, 2) fast3d_kernel(const __grid_constant__ F
   };
   const Coef<T> cf{(T)g.k0, (T)g.k1};
   const int tid = threadIdx.x;
-  const int zg = tid >> 6, lp = (tid >> 3) & 7, xq = tid & 7;  // row group, line pair, col quad
+  const int zg = tid / (NLP * 8), lp = (tid >> 3) % NLP, xq = tid & 7;  // row group (= warp for NY=8), line pair, col quad
   const int64_t ns0 = g.S0_hi - g.S0_lo + 1;
   const int64_t n1 = g.n1, n2 = g.n2, n_items = ns0 * n1 * n2;
   const int64_t plane = g.N1 * g.N2;
@@ -149,6 +159,14 @@ __global__ void __launch_bounds__(NT, 2) fast3d_kernel(const __grid_constant__ F
       item_s[0] = S0;
       item_s[1] = q1;
       item_s[2] = q2;
+      if (g.trace && it < n_items) {
+        unsigned smid;
+        asm volatile("mov.u32 %0, %smid;" : "=r"(smid));
+        g.trace[it * kTraceStride] = ((long long)smid << 32) | (long long)(q1 * 65536 + q2);
+        g.trace[it * kTraceStride + 1] = gtimer();
+        item_s[0] = S0;
+      }
+      trace_it_s = it;
     }
     __syncthreads();
     const int64_t S0 = item_s[0];
@@ -173,8 +191,11 @@ __global__ void __launch_bounds__(NT, 2) fast3d_kernel(const __grid_constant__ F
       mbar_wait_parity(&mbar[ib], phase[ib]);
       phase[ib] ^= 1u;
     }
+    long long* tr = (g.trace && tid == 0) ? g.trace + trace_it_s * kTraceStride : nullptr;
+    if (tr) tr[2] = gtimer();
 
     for (int a = g.a_lo; a <= g.a_hi; ++a) {
+      const int tk = 3 + 3 * (a - g.a_lo);
       const int ib = a & 1, ob = (a + 1) & 1;
       if (a > g.a_lo) {
         const int plo = g.lo[a - 1], phi = g.hi[a - 1];  // rows computed at level a-1
@@ -187,6 +208,7 @@ __global__ void __launch_bounds__(NT, 2) fast3d_kernel(const __grid_constant__ F
             while (ld_acquire(g.flags + fbase + q1 * n2 + q2 - 1) < need) __nanosleep(20);
           if (q1 > 0 && q2 > 0)
             while (ld_acquire(g.flags + fbase + (q1 - 1) * n2 + q2 - 1) < need) __nanosleep(20);
+          if (tr) tr[tk] = gtimer();
           fence_proxy_async_smem();
           mbar_arrive_expect_tx(&mbar[ib], (cline_bytes + ccol_bytes) * (phi - plo + 1));
           const int par = (int)((g.tau0 + a) & 1);
@@ -199,6 +221,7 @@ __global__ void __launch_bounds__(NT, 2) fast3d_kernel(const __grid_constant__ F
         }
         mbar_wait_parity(&mbar[ib], phase[ib]);  // carries + the In planes issued at level a-1
         phase[ib] ^= 1u;
+        if (tr) tr[tk + 1] = gtimer();
         // the CL carry columns of each computed plane into place
         const int nc = phi - plo + 1;
         for (int e = tid; e < nc * NY * CL; e += NT) {
@@ -226,11 +249,17 @@ __global__ void __launch_bounds__(NT, 2) fast3d_kernel(const __grid_constant__ F
       const int mid = (rlo + rhi) >> 1;
       const int r0 = zg == 0 ? rlo : mid + 1, r1 = zg == 0 ? mid : rhi;
       const int64_t yb = Y0 - a + 2 * lp, xb = X0 - SIGMA * a + 1 + 4 * xq;  // output (0, 0)
-      bool lineok[2], colok[4];
+      // per-output masks (bit i*4+j): interior in (y, x); successors' carry cells
+      uint32_t vmask = 0, cmask = 0;
 #pragma unroll
-      for (int i = 0; i < 2; ++i) lineok[i] = (yb + i >= 1) && (yb + i <= g.N1 - 2);
+      for (int i = 0; i < 2; ++i)
 #pragma unroll
-      for (int j = 0; j < 4; ++j) colok[j] = (xb + j >= 1) && (xb + j <= g.N2 - 2);
+        for (int j = 0; j < 4; ++j) {
+          const bool ok = (yb + i >= 1) && (yb + i <= g.N1 - 2) && (xb + j >= 1) && (xb + j <= g.N2 - 2);
+          const bool carry = (lp == NLP - 1) || (4 * xq + j >= NX - CL);
+          vmask |= (ok ? 1u : 0u) << (i * 4 + j);
+          cmask |= (ok && carry ? 1u : 0u) << (i * 4 + j);
+        }
       T* dst = static_cast<T*>(g.buf[(g.tau0 + a + 1) & 1]);
       const bool fin = (a == g.a_final);
 
@@ -254,6 +283,7 @@ __global__ void __launch_bounds__(NT, 2) fast3d_kernel(const __grid_constant__ F
       auto step = [&](int r, const T (&P)[4][6], const T (&C)[4][6], const T (&N)[4][6]) {
         const int64_t z = i0 + r;
         const bool zok = (z >= 1) && (z <= g.N0 - 2);
+        const uint32_t okm = zok ? vmask : 0u;
         T out[2][4];
 #pragma unroll
         for (int i = 0; i < 2; ++i)
@@ -269,7 +299,7 @@ __global__ void __launch_bounds__(NT, 2) fast3d_kernel(const __grid_constant__ F
                 x[2][dy][dx] = N[i + dy][j + dx];
               }
             const T v = apply<T, KIND>(x, cf);
-            out[i][j] = (zok && lineok[i] && colok[j]) ? v : x[1][1][1];
+            out[i][j] = ((okm >> (i * 4 + j)) & 1u) ? v : x[1][1][1];
           }
         // into the output buffer: columns CL + 4xq + j (one scalar, one pair, one scalar)
 #pragma unroll
@@ -286,14 +316,14 @@ __global__ void __launch_bounds__(NT, 2) fast3d_kernel(const __grid_constant__ F
         if (a == g.H) full = full || r == rlo || r == rhi;
         else if (a > g.H && a < g.L - 1) full = full || r <= rlo + 1 || r >= rhi - 1;
         else if (a == g.L - 1) full = true;
-        if (zok) {
-          T* zp = dst + z * plane;
+        const uint32_t sm_ = zok ? (full ? vmask : cmask) : 0u;
+        if (sm_) {
+          T* rp = dst + z * plane + yb * g.N2 + xb;
 #pragma unroll
           for (int i = 0; i < 2; ++i)
 #pragma unroll
             for (int j = 0; j < 4; ++j)
-              if (lineok[i] && colok[j] && (full || lp == 7 || 4 * xq + j >= NX - CL))
-                zp[(yb + i) * g.N2 + xb + j] = out[i][j];
+              if ((sm_ >> (i * 4 + j)) & 1u) rp[i * g.N2 + j] = out[i][j];
         }
       };
 
@@ -316,6 +346,7 @@ __global__ void __launch_bounds__(NT, 2) fast3d_kernel(const __grid_constant__ F
         }
       }
       __syncthreads();  // level a complete in ob; every thread's stores of level a issued
+      if (tr) tr[tk + 2] = gtimer();
       if (tid == 0) {
         __threadfence();
         st_release(my_flag, a - g.a_lo + 1);
@@ -349,8 +380,13 @@ static bool encode(CUtensorMap* map, void* base, const Fast3DArgs& a, uint32_t b
             CU_TENSOR_MAP_L2_PROMOTION_L2_128B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE) == CUDA_SUCCESS;
 }
 
+static long long* g_trace = nullptr;
+static int64_t g_trace_launch = -1, g_launch_count = 0;
+
 template <typename T, int KIND>
-cudaError_t launch_t(const Fast3DArgs& a, cudaStream_t s) {
+cudaError_t launch_t(const Fast3DArgs& a_in, cudaStream_t s) {
+  Fast3DArgs a = a_in;
+  a.trace = (g_trace && g_launch_count++ == g_trace_launch) ? g_trace : nullptr;
   static int grid = 0;
   static size_t attr_bytes = 0;
   const size_t smem = smem_bytes<T>(a.Q);
@@ -379,6 +415,12 @@ cudaError_t launch_t(const Fast3DArgs& a, cudaStream_t s) {
 
 }  // namespace fast3d
 
+void fast3d_set_trace(long long* dev_buf, int64_t launch_index) {
+  fast3d::g_trace = dev_buf;
+  fast3d::g_trace_launch = launch_index;
+  fast3d::g_launch_count = 0;
+}
+
 size_t fast3d_smem_bytes(int dtype, int Q) {
   return dtype == 1 ? fast3d::smem_bytes<double>(Q) : fast3d::smem_bytes<float>(Q);
 }
@@ -397,3 +439,8 @@ cudaError_t launch_fast3d(int variant, const Fast3DArgs& a, int /*grid: persiste
 }
 
 }  // namespace hexs
+
+// Debug hook (not part of include/stencil.h): trace one 3D launch's per-item timeline.
+extern "C" void hexs_debug_fast3d_trace(void* dev_buf, int64_t launch_index) {
+  hexs::fast3d_set_trace(static_cast<long long*>(dev_buf), launch_index);
+}

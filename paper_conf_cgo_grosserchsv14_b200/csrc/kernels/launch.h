@@ -82,10 +82,13 @@ struct Fast3DArgs {
   double k0, k1;
   int* flags;
   unsigned long long* counter;
+  long long* trace;  // optional (debug): per-item timestamps, see hex3d.cu
   int32_t lo[kMaxH], hi[kMaxH];
 };
+// Debug tracing of the 3D kernel (host-set device buffer; NULL disables).
+void fast3d_set_trace(long long* dev_buf, int64_t n_items_cap);
 cudaError_t launch_fast3d(int variant, const Fast3DArgs& a, int grid, cudaStream_t s);
-constexpr int kFast3DNY = 16, kFast3DNX = 32;  // classical tile of the 3D fast kernel
+constexpr int kFast3DNY = 8, kFast3DNX = 32;  // classical tile of the 3D fast kernel
 size_t fast3d_smem_bytes(int dtype, int Q);
 
 }  // namespace hexs
