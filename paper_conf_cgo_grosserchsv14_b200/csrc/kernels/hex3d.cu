@@ -346,11 +346,10 @@ __global__ void __launch_bounds__(NT, MINB) fast3d_kernel(const __grid_constant_
         }
       }
       __syncthreads();  // level a complete in ob; every thread's stores of level a issued
+      // st.release.gpu after the CTA barrier is cumulative over the barrier-ordered stores of
+      // every thread of the CTA (PTX memory model), so no separate membar is needed
+      if (tid == 0) st_release(my_flag, a - g.a_lo + 1);
       if (tr) tr[tk + 2] = gtimer();
-      if (tid == 0) {
-        __threadfence();
-        st_release(my_flag, a - g.a_lo + 1);
-      }
     }
   }
 }

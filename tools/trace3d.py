@@ -33,3 +33,4 @@ for k in range(L_):
         k, (f - prev)[ok].mean(), (d - f)[ok].mean(), (c - d)[ok].mean()))
 tot = rel[:, 4 + 3 * (L_ - 1)] - rel[:, 0]
 print("per item total us: mean %.2f; items per CTA-slot %.1f" % (tot.mean(), n / 296))
+np.save(os.path.join(os.path.dirname(os.path.dirname(os.path.abspath(__file__))), "gpurun_out", "trace3d.npy"), t)
