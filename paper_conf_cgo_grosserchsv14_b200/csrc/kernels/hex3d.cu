@@ -111,11 +111,11 @@ __device__ __forceinline__ T apply(const T (&x)[3][3][3], const Coef<T>& k) {
 template <typename T, int KIND>
 __global__ void __launch_bounds__(NT, MINB) fast3d_kernel(const __grid_constant__ Fast3DArgs g,
                                                        const __grid_constant__ Maps m) {
-  extern __shared__ __align__(128) unsigned char smem_raw[];
+  extern __shared__ __align__(1024) unsigned char smem_raw[];  // dynamic base is 1024-B aligned
   __shared__ __align__(8) uint64_t mbar[2];
   __shared__ int64_t item_s[3];
   __shared__ int64_t trace_it_s;
-  T* buf = reinterpret_cast<T*>((reinterpret_cast<uintptr_t>(smem_raw) + 127) & ~uintptr_t(127));
+  T* buf = reinterpret_cast<T*>(smem_raw);  // stays a shared-space pointer (LDS/STS, not generic LD/ST)
   T* side = buf + (size_t)2 * g.Q * PP<T>;  // [Q][NY][CW] landing area of the carry columns
   auto B = [&](int which, int q, int ly, int lx) -> T* {
     return buf + ((size_t)which * g.Q + q) * PP<T> + ly * SX + lx;
