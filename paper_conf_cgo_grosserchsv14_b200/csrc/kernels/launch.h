@@ -83,6 +83,7 @@ struct Fast3DArgs {
   int* flags;
   unsigned long long* counter;
   long long* trace;  // optional (debug): per-item timestamps, see hex3d.cu
+  int dbg;           // debug timing modes (0 in production), see hex3d.cu
   int32_t lo[kMaxH], hi[kMaxH];
 };
 // Debug tracing of the 3D kernel (host-set device buffer; NULL disables).
