@@ -52,7 +52,7 @@ def _units():
     units = []
     for src in ["desc.cpp", "plan.cpp"]:
         units.append((os.path.join(CSRC, src), "cxx", []))
-    for src in ["run.cu", "kernels/generic.cu", "kernels/registry.cu", "kernels/hex3d.cu"]:
+    for src in ["run.cu", "kernels/generic.cu", "kernels/registry.cu", "kernels/hex3d.cu", "kernels/fdtd.cu"]:
         units.append((os.path.join(CSRC, src), "nvcc", []))
     for vid in _variant_ids("fast2d_variants.h", "HEXS_FAST2D_VARIANTS"):
         units.append((os.path.join(KDIR, "fast2d_inst.cu"), "nvcc", [f"-DHEXS_VARIANT={vid}"]))

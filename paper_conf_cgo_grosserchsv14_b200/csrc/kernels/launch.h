@@ -57,7 +57,8 @@ struct Fast2DArgs {
 };
 cudaError_t launch_fast2d(int variant, const Fast2DArgs& a, int grid, cudaStream_t s);
 
-// FDTD-2D fast kernel.
+// FDTD-2D fast kernel (kernels/fdtd.cu): one CTA per hexagon, j streamed through a
+// shared-memory ring.
 struct FdtdArgs {
   void* f[3];  // ex, ey, hz
   int64_t N0, N1;
@@ -66,8 +67,10 @@ struct FdtdArgs {
   int64_t S0_lo, row_off;
   int W;
   double k0, k1;
+  int32_t lo[kMaxH], hi[kMaxH];  // hexagon rows per level
 };
 cudaError_t launch_fdtd(int variant, const FdtdArgs& a, int grid, cudaStream_t s);
+size_t fdtd_smem_bytes(int dtype, int W);
 
 // 3D fast kernel.
 // 3D fast kernel (wavefront of smem-resident classical tiles, kernels/hex3d.cu).

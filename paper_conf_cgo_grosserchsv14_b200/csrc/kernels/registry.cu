@@ -38,9 +38,13 @@ cudaError_t launch_fast2d(int variant, const Fast2DArgs& a, int grid, cudaStream
   }
 }
 
-// Not yet specialised: FDTD-2D and 3D classes run the generic hybrid kernel.
-int fdtd_variant(int, int, int) { return -1; }
-cudaError_t launch_fdtd(int, const FdtdArgs&, int, cudaStream_t) { return cudaErrorInvalidValue; }
+// FDTD-2D fast kernel: any (h, w0) whose hexagon (W = 2 w0 + 2 + h + floor(h/2) rows, delta0
+// = 1, delta1 = 1/2) fits the shared-memory ring and whose 2h+2 levels fit one ring block.
+int fdtd_variant(int dtype, int h, int w0) {
+  const int W = 2 * w0 + 2 + h + h / 2;
+  if (2 * h + 2 > 64 || fdtd_smem_bytes(dtype, W) > 200 * 1024) return -1;
+  return dtype == 1 ? 1 : 0;
+}
 // 3D fast kernel: any (h, w0) whose two level buffers fit in shared memory
 // (2 * (w0 + 2h + 3) planes x 18 lines x 40 columns).
 int fast3d_variant(int kind, int dtype, int h, int w0) {

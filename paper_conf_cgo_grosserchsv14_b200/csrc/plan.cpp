@@ -208,7 +208,8 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
   } else if (flags == STENCIL_EXEC_AUTO) {
     if (d.kind == STENCIL_FDTD2D) {
       p->variant = fdtd_variant(dtype, h, w0);
-      if (p->variant >= 0 && p->hd == 0) ex = EXEC_FDTD;
+      // the ring is filled by 16-B cp.async: row starts must be 16-B aligned
+      if (p->variant >= 0 && p->hd == 0 && (d.ext[1] * (int64_t)d.elem()) % 16 == 0) ex = EXEC_FDTD;
     } else if (d.dims == 2) {
       p->variant = fast2d_variant(d.kind, dtype, h, w0);
       if (p->variant >= 0 && p->hd == 0 && p->dcls[0] == 1 && p->d0.n == 1 && p->d0.d == 1 &&

@@ -151,6 +151,10 @@ stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* 
         a.W = p.W;
         a.k0 = d.coef[0];
         a.k1 = d.coef[1];
+        for (int q = 0; q < p.H; ++q) {
+          a.lo[q] = p.lo[q];
+          a.hi[q] = p.hi[q];
+        }
         HEXS_CUDA(launch_fdtd(p.variant, a, grid, s), "stencil_run: fdtd kernel launch");
       } else if (p.executor == EXEC_FAST3D) {
         Fast3DArgs a{};

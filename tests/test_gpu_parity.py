@@ -108,6 +108,21 @@ def test_fdtd(dtype, executor):
             assert_bitexact(a, b, f"fdtd {name} {executor} {shape}")
 
 
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("shape,T,h,w0", [((64, 80), 9, 0, 0), ((101, 260), 17, 0, 0), ((37, 132), 13, 2, 0),
+                                          ((90, 72), 11, 5, 3), ((70, 200), 25, 3, 1), ((130, 68), 8, 8, 4),
+                                          ((9, 4), 5, 0, 0), ((300, 324), 30, 5, 5)])
+def test_fdtd_fast_kernel(dtype, shape, T, h, w0):
+    """The shared-memory-ring FDTD kernel (kernels/fdtd.cu): ragged chunk tails, hexagons cut
+    by the grid, partial first/last launches, tiny grids -- bit-exact against the oracle."""
+    f = stencil_inputs.fields(shape, seed=22, n=3, dtype=dtype)
+    got, plan = _gpu_fdtd(f, T, dtype, h=h, w0=w0)
+    assert plan.info["fast_kernel"] == 1
+    exp = oracle.fdtd(*f, T)
+    for name, a, b in zip(("ex", "ey", "hz"), got, exp):
+        assert_bitexact(a, b, f"fdtd fast {name} {shape} h={h} w0={w0}")
+
+
 @pytest.mark.parametrize("h,w0", [(2, 0), (5, 3), (3, 1)])
 def test_fdtd_tiles(h, w0):
     f = stencil_inputs.fields((90, 70), seed=21, n=3)
