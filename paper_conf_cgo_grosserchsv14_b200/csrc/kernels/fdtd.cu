@@ -16,8 +16,10 @@
 //     (LDGSTS, every address 16-B aligned -- the aligned loads of Sec. 4.2.3), so no warp
 //     waits on HBM latency; out-of-grid chunks are zero-filled and never used;
 //   * a level is a pure map over its cells (each statement reads only the other fields and
-//     its own old value), so one CTA barrier separates levels; two threads per column split
-//     the rows;
+//     its own old value), so one CTA barrier separates levels; four threads per column split
+//     the rows (interleaved, so a warp is 32 consecutive columns of one row: conflict-free);
+//     the fields are disjoint ring regions (__restrict__), so a thread's row loads are
+//     batched ahead of its stores;
 //   * a column is final once no later chunk touches it (j < (k+1)C - a_hi): after each chunk
 //     its C final columns of every row the hexagon modifies are written back with coalesced
 //     stores -- the interleaved copy-out of Sec. 4.2.1.
@@ -31,7 +33,8 @@ namespace fdtd {
 
 constexpr int C = 64;        // columns per chunk (= ring block)
 constexpr int RC = 4 * C;    // ring columns
-constexpr int NT = 2 * C;    // two threads per column
+constexpr int RP = 4;        // threads per column (row parts, rows interleaved)
+constexpr int NT = RP * C;
 
 template <typename T>
 size_t smem_bytes(int W) {
@@ -54,7 +57,7 @@ __device__ __forceinline__ int64_t min64(int64_t a, int64_t b) { return a < b ? 
 
 // fields: 0 = ex, 1 = ey, 2 = hz (the order of FdtdArgs::f); statement k: 0 ey, 1 ex, 2 hz
 template <typename T>
-__global__ void __launch_bounds__(NT) fdtd_kernel(const __grid_constant__ FdtdArgs g) {
+__global__ void __launch_bounds__(NT, 2) fdtd_kernel(const __grid_constant__ FdtdArgs g) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
   T* ring = reinterpret_cast<T*>(smem_raw);
   const int W = g.W, R = W + 2;  // smem rows: b in [-1, W] at b + 1
@@ -91,82 +94,102 @@ __global__ void __launch_bounds__(NT) fdtd_kernel(const __grid_constant__ FdtdAr
   constexpr int RSTEP = NT / NCH;
   static_assert(NT % NCH == 0, "staging walk");
   const int sc = tid % NCH;
-  auto stage = [&](int64_t blk) {
-    const int64_t j = (blk - 1) * C + sc * CH;
+  // A thread stages the same (field, row) pairs for every block: fr = tid/NCH + u*RSTEP.
+  // Their row base pointers (NULL outside the grid) are computed once.
+  constexpr int MAXU = (3 * 42 + RSTEP - 1) / RSTEP;  // ceil(3 (W+2) / RSTEP) for W <= 40 (fdtd_variant)
+  const T* rowp[MAXU];
+  int soff[MAXU];
+#pragma unroll
+  for (int u = 0; u < MAXU; ++u) {
+    const int fr = tid / NCH + u * RSTEP;
+    const int f = fr / R, rb = fr - f * R;
+    const int64_t i = i0 + rb - 1;
+    const bool ok = fr < 3 * R && i >= 0 && i < N0;
+    T* const fb = f == 0 ? F[0] : (f == 1 ? F[1] : F[2]);
+    rowp[u] = ok ? fb + i * N1 : nullptr;
+    soff[u] = fr < 3 * R ? (f * R + rb) * RC : -1;
+  }
+  auto stage = [&](int blk) {
+    const int j = (blk - 1) * C + sc * CH;
     const bool jok = j >= 0 && j < N1;
-    const int cj = (int)((j + C) & (RC - 1));
-    int f = 0, rb = tid / NCH;  // smem row index (b + 1) within field f
-    for (int fr = tid / NCH; fr < 3 * R; fr += RSTEP) {
-      while (rb >= R) rb -= R, ++f;
-      const int64_t i = i0 + rb - 1;
-      const bool ok = jok && i >= 0 && i < N0;
-      const T* base = f == 0 ? F[0] : (f == 1 ? F[1] : F[2]);
-      const T* src = ok ? base + i * N1 + j : base;
-      cp_async16(ring + ((size_t)f * R + rb) * RC + cj, src, ok);
-      rb += RSTEP;
+    const int cj = (j + C) & (RC - 1);
+#pragma unroll
+    for (int u = 0; u < MAXU; ++u) {
+      if (soff[u] < 0) continue;
+      const bool ok = jok && rowp[u] != nullptr;
+      cp_async16(ring + soff[u] + cj, ok ? rowp[u] + j : F[0], ok);
     }
     cp_async_commit();
   };
 
-  const int64_t k_last = (N1 - 1 + g.a_hi) / C;
+  // per level (relative index a - a_lo): statement, rows [blo, bhi] clipped to the grid and
+  // the statement's domain (oracle/oracle.c: ey i >= 1; ex j >= 1; hz i < N0-1, j < N1-1),
+  // column range [jlo, jhi] of the statement
+  __shared__ int lv[kMaxH][5];
+  const int nlev = g.a_hi - g.a_lo + 1;
+  if (tid < nlev) {
+    const int a = g.a_lo + tid;
+    const int st = (int)((g.tau0 + a) % 3);
+    const int64_t ilo = st == 0 ? 1 : 0, ihi = st == 2 ? N0 - 2 : N0 - 1;
+    lv[tid][0] = st;
+    lv[tid][1] = (int)max64(g.lo[a], ilo - i0);
+    lv[tid][2] = (int)min64(g.hi[a], ihi - i0);
+    lv[tid][3] = st == 1 ? 1 : 0;
+    lv[tid][4] = (int)(st == 2 ? N1 - 2 : N1 - 1);
+  }
+  const int k_last = (int)((N1 - 1 + g.a_hi) / C);
   stage(0);
   stage(1);
   stage(2);
-  const int col = tid & (C - 1), rpar = tid / C;
+  const int col = tid & (C - 1), rpar = tid / C;  // column, row part
   T* const rex = ring + (size_t)(0 * R + 1) * RC;  // row b of a field at r.. + b * RC + ring column
   T* const rey = ring + (size_t)(1 * R + 1) * RC;
   T* const rhz = ring + (size_t)(2 * R + 1) * RC;
-  for (int64_t k = 0; k <= k_last; ++k) {
+  for (int k = 0; k <= k_last; ++k) {
     stage(k + 3);          // next chunk's new block (ring slot of block k-1, written back)
     cp_async_wait<1>();    // every block but the newest has landed
     __syncthreads();
-    for (int a = g.a_lo; a <= g.a_hi; ++a) {
-      const int st = (int)((g.tau0 + a) % 3);
-      const int64_t j = k * C - a + col;
-      const int cj = (int)((j + C) & (RC - 1));
-      // statement domains (oracle/oracle.c): ey i >= 1; ex j >= 1; hz i < N0-1, j < N1-1
-      const int64_t ilo = st == 0 ? 1 : 0, ihi = st == 2 ? N0 - 2 : N0 - 1;
-      const bool jok = st == 1 ? (j >= 1 && j < N1) : (st == 2 ? (j >= 0 && j < N1 - 1) : (j >= 0 && j < N1));
-      const int blo = (int)max64(g.lo[a], ilo - i0), bhi = (int)min64(g.hi[a], ihi - i0);
-      if (jok) {
-        int b = blo + rpar;
+    for (int l = 0; l < nlev; ++l) {
+      const int st = lv[l][0], blo = lv[l][1], bhi = lv[l][2];
+      const int j = k * C - (g.a_lo + l) + col;
+      if (j >= lv[l][3] && j <= lv[l][4]) {
+        const int cj = (j + C) & (RC - 1);
+        const int b0 = blo + rpar;
         if (st == 0) {  // ey[i][j] -= ce * (hz[i][j] - hz[i-1][j])
-          T* pe = rey + b * RC + cj;
-          const T* ph = rhz + b * RC + cj;
-#pragma unroll 2
-          for (; b <= bhi; b += 2, pe += 2 * RC, ph += 2 * RC) *pe = fdtd_ey<T>(*pe, ph[0], ph[-RC], cf);
+          T* __restrict__ pe = rey + cj + b0 * RC;
+          const T* __restrict__ ph = rhz + cj + b0 * RC;
+#pragma unroll 4
+          for (int b = b0; b <= bhi; b += RP, pe += RP * RC, ph += RP * RC) *pe = fdtd_ey<T>(*pe, ph[0], ph[-RC], cf);
         } else if (st == 1) {  // ex[i][j] -= ce * (hz[i][j] - hz[i][j-1])
-          const int cjm = (int)((j - 1 + C) & (RC - 1));
-          T* px = rex + b * RC + cj;
-          const T* ph = rhz + b * RC + cj;
-          const T* phm = rhz + b * RC + cjm;
-#pragma unroll 2
-          for (; b <= bhi; b += 2, px += 2 * RC, ph += 2 * RC, phm += 2 * RC) *px = fdtd_ex<T>(*px, *ph, *phm, cf);
+          const int dm = ((j - 1 + C) & (RC - 1)) - cj;  // column j-1 relative to j in the ring
+          T* __restrict__ px = rex + cj + b0 * RC;
+          const T* __restrict__ ph = rhz + cj + b0 * RC;
+#pragma unroll 4
+          for (int b = b0; b <= bhi; b += RP, px += RP * RC, ph += RP * RC) *px = fdtd_ex<T>(*px, ph[0], ph[dm], cf);
         } else {  // hz[i][j] -= ch * (((ex[i][j+1] - ex[i][j]) + ey[i+1][j]) - ey[i][j])
-          const int cjp = (int)((j + 1 + C) & (RC - 1));
-          T* ph = rhz + b * RC + cj;
-          const T* px = rex + b * RC + cj;
-          const T* pxp = rex + b * RC + cjp;
-          const T* pe = rey + b * RC + cj;
-#pragma unroll 2
-          for (; b <= bhi; b += 2, ph += 2 * RC, px += 2 * RC, pxp += 2 * RC, pe += 2 * RC)
-            *ph = fdtd_hz<T>(*ph, *pxp, *px, pe[RC], pe[0], cf);
+          const int dp = ((j + 1 + C) & (RC - 1)) - cj;  // column j+1 relative to j in the ring
+          T* __restrict__ ph = rhz + cj + b0 * RC;
+          const T* __restrict__ px = rex + cj + b0 * RC;
+          const T* __restrict__ pe = rey + cj + b0 * RC;
+#pragma unroll 4
+          for (int b = b0; b <= bhi; b += RP, ph += RP * RC, px += RP * RC, pe += RP * RC)
+            *ph = fdtd_hz<T>(*ph, px[dp], px[0], pe[RC], pe[0], cf);
         }
       }
       __syncthreads();
     }
     // write back the columns no later chunk touches: [kC - a_hi, (k+1)C - a_hi), or all
     // remaining columns after the last chunk
-    const int64_t wlo = max64(0, k * C - g.a_hi);
-    const int64_t whi = (k == k_last) ? N1 - 1 : (k + 1) * C - g.a_hi - 1;
-    for (int64_t j = k * C - g.a_hi + col; j <= whi; j += C) {
+    const int wlo = max(0, k * C - g.a_hi);
+    const int whi = (k == k_last) ? (int)N1 - 1 : (k + 1) * C - g.a_hi - 1;
+    for (int j = k * C - g.a_hi + col; j <= whi; j += C) {
       if (j < wlo) continue;
-      const int cj = (int)((j + C) & (RC - 1));
+      const int cj = (j + C) & (RC - 1);
 #pragma unroll
       for (int f = 0; f < 3; ++f) {
         const T* sp = (f == 0 ? rex : (f == 1 ? rey : rhz)) + cj;
-        T* gp = F[f] + j;
-        for (int b = mlo[f] + rpar; b <= mhi[f]; b += 2) gp[(i0 + b) * N1] = sp[b * RC];
+        T* gp = F[f] + (i0 * N1 + j);
+        for (int b = mlo[f] + rpar; b <= mhi[f]; b += RP) gp[b * N1] = sp[b * RC];
       }
     }
     __syncthreads();  // the write-back reads ring slots the next stage() overwrites

@@ -42,7 +42,7 @@ cudaError_t launch_fast2d(int variant, const Fast2DArgs& a, int grid, cudaStream
 // = 1, delta1 = 1/2) fits the shared-memory ring and whose 2h+2 levels fit one ring block.
 int fdtd_variant(int dtype, int h, int w0) {
   const int W = 2 * w0 + 2 + h + h / 2;
-  if (2 * h + 2 > 64 || fdtd_smem_bytes(dtype, W) > 200 * 1024) return -1;
+  if (2 * h + 2 > 64 || W > 40 || fdtd_smem_bytes(dtype, W) > 200 * 1024) return -1;
   return dtype == 1 ? 1 : 0;
 }
 // 3D fast kernel: any (h, w0) whose two level buffers fit in shared memory

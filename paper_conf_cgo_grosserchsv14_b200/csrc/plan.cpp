@@ -18,9 +18,21 @@
 #include <set>
 #include <string>
 
+#include <cuda_runtime.h>
+
 #include "internal.h"
 
 namespace hexs {
+
+// SMs of the current device (148 on B200 when no device is visible, e.g. planning on a host)
+static int device_sm_count() {
+  int dev = 0, sms = 0;
+  if (cudaGetDevice(&dev) == cudaSuccess && cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev) == cudaSuccess &&
+      sms > 0)
+    return sms;
+  cudaGetLastError();
+  return 148;
+}
 
 namespace {
 
@@ -162,7 +174,15 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
   const int dtype = d.dtype;
   if (auto_tile) {
     if (d.kind == STENCIL_FDTD2D) {
-      h = 5; w0 = 8;  // 12 tau-levels = 4 full steps per tile (h+1 multiple of 3)
+      // 24 tau-levels = 8 full steps per tile (h+1 a multiple of 3, reading R14); w0 as
+      // small as possible while every launch's hexagons (W = 2 w0 + 2 + h + h/2 rows) fit one
+      // wave of the FDTD kernel (2 CTAs per SM): a second, partial wave would double the
+      // launch time (grid quantisation).  Best measured on B200: profiles/round1/.
+      h = 11;
+      w0 = 5;
+      const int64_t slots = 2 * (int64_t)device_sm_count();
+      auto Wof = [&](int w) { return (int64_t)2 * w + 2 + h + h / 2; };
+      while (w0 < 12 && (d.ext[0] + Wof(w0) - 1) / Wof(w0) + 1 > slots) ++w0;
     } else if (d.dims == 2) {
       h = 3; w0 = 7;  // best measured on B200 (profiles/)
     } else {

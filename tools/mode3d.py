@@ -1,8 +1,5 @@
-"""Timing experiment for the fast 3D kernel: python tools/mode3d.py [h w0].
-
-Runs the heat3d config with the kernel's debug modes (0 = normal, 1 = no carries,
-2 = no In planes, 3 = neither; results are WRONG in modes 1-3) to split the step time
-into compute-bound and load/handoff-bound parts."""
+"""Timing experiment for the fast 3D kernel: python tools/mode3d.py [config [h w0]].
+Mode 1 skips the progress counters (results are WRONG) to measure the synchronisation cost."""
 import ctypes
 import os
 import sys
@@ -13,18 +10,17 @@ import torch  # noqa: E402
 import bench  # noqa: E402
 from paper_conf_cgo_grosserchsv14_b200 import Plan, Stencil, lib  # noqa: E402
 
-tile = {}
-if len(sys.argv) > 2:
-    tile = {"h": int(sys.argv[1]), "w0": int(sys.argv[2])}
-kind, ext, T, _ = bench.CONFIGS["heat3d"]
+cfg = sys.argv[1] if len(sys.argv) > 1 else "heat3d"
+tile = {"h": int(sys.argv[2]), "w0": int(sys.argv[3])} if len(sys.argv) > 3 else {}
+kind, ext, T, _ = bench.CONFIGS[cfg]
 g = bench.make_inputs(kind, ext)[0]
 plan = Plan(Stencil(kind, ext), T, **tile)
 x = torch.from_numpy(g).cuda()
 o = torch.empty_like(x)
 L = lib()
 L.hexs_debug_fast3d_mode.argtypes = [ctypes.c_int]
-ups = float(g.size) * T
-for mode in [int(m) for m in os.environ.get('MODES', '0 1 2 3 0').split()]:
+ups = plan.info["updates"]
+for mode in [int(m) for m in os.environ.get("MODES", "0 1 0").split()]:
     L.hexs_debug_fast3d_mode(mode)
     plan.run(x, o)
     torch.cuda.synchronize()
@@ -35,5 +31,5 @@ for mode in [int(m) for m in os.environ.get('MODES', '0 1 2 3 0').split()]:
     e.record()
     torch.cuda.synchronize()
     ms = s.elapsed_time(e) / 3
-    print("mode %d: %.2f ms/run  %.0f GUp/s" % (mode, ms, ups / ms / 1e6))
+    print("%s h,w0=%s mode %d: %.2f ms/run  %.0f GUp/s" % (cfg, tile, mode, ms, ups / ms / 1e6), flush=True)
 L.hexs_debug_fast3d_mode(0)
