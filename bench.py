@@ -103,10 +103,60 @@ class ClockSampler:
                 "samples": len(sm)}
 
 
-def bytes_per_update_tiled(info, word):
+def fdtd_hexagon_traffic(lo, hi):
+    """FDTD-2D In/Out sets of one full hexagon per classical column, over all three fields
+    (statement k = tau mod 3 writes ey, ex, hz; PolyBench reads, R9).  A read is In
+    when the version it reads (the last write of that field and row before its level) lies
+    outside the hexagon; a write is Out when a reader of that version (levels a+1..a+3, every
+    statement also reads its own old value) lies outside.  Returns (tau-points, In, Out)."""
+    H = len(lo)
+    inside = lambda a, b: 0 <= a < H and lo[a] <= b <= hi[a]
+    writes = {0: "ey", 1: "ex", 2: "hz"}
+    reads = {0: [("hz", 0), ("hz", -1), ("ey", 0)], 1: [("hz", 0), ("ex", 0)],
+             2: [("ex", 0), ("ey", 1), ("ey", 0), ("hz", 0)]}
+    kof = {"ey": 0, "ex": 1, "hz": 2}
+    ins, outs, pts = set(), 0, 0
+    for a in range(H):
+        for b in range(lo[a], hi[a] + 1):
+            pts += 1
+            for f, d in reads[a % 3]:
+                ap = a - 1
+                while ap % 3 != kof[f]:
+                    ap -= 1
+                if not inside(ap, b + d):
+                    ins.add((f, b + d, ap))
+            f = writes[a % 3]
+            outs += any(f2 == f and not inside(a2, b - d)
+                        for a2 in range(a + 1, a + 4) for f2, d in reads[a2 % 3])
+    return pts, len(ins), outs
+
+
+def bytes_per_update_tiled(info, word, plan=None):
     """Algorithmic HBM bytes per update of the hybrid schedule: word*(In+Out)/points of the
-    plan's full hexagon per classical column (DESIGN.md roofline)."""
+    plan's full hexagon per classical column.  FDTD: per point-step (three
+    tau-points), In/Out over all three fields."""
+    if plan is not None and plan.stencil.kind == "fdtd2d":
+        lo, hi = plan.hexagon()
+        pts, n_in, n_out = fdtd_hexagon_traffic(lo, hi)
+        return word * (n_in + n_out) / (pts / 3)
     return word * (info["tile_in"] + info["tile_out"]) / info["tile_points"]
+
+
+KERNEL_NAMES = {"fast2d": "fast2d_kernel (2D register wavefront)", "fdtd": "fdtd_kernel (FDTD smem ring)",
+                "fast3d": "fast3d_kernel (3D classical-tile wavefront)", "generic": "generic_kernel"}
+
+
+def measured_traffic(cfg, tile):
+    """DRAM bytes per launch of the phase kernel from the committed ncu launch list
+    (profiles/round1/traffic_<cfg>.json: dram__bytes_read.sum + dram__bytes_write.sum summed
+    over every launch of one stencil_run, divided by the launch count), or None."""
+    p = os.path.join(ROOT, "profiles", "round1", f"traffic_{cfg}.json")
+    if not os.path.exists(p):
+        return None
+    d = json.load(open(p))
+    if d.get("tile") != tile:
+        return None
+    return d["dram_bytes_per_launch"]
 
 
 def cpu_baseline(kind, ext, target_s=12.0):
@@ -239,7 +289,7 @@ def run_gpu(args, cfg):
     prof = plan.profile_read()
     plan.profile(0)
     word = 4
-    bpu = bytes_per_update_tiled(info, word)
+    bpu = bytes_per_update_tiled(info, word, plan)
     n_launch_per_step = info["n_launches"]
     avg_launch_ms = prof["kernel_ms"] / prof["launches"]
     # algorithmic bytes of one average launch = updates per launch x bytes/update
@@ -281,8 +331,12 @@ def run_gpu(args, cfg):
                    "tile": {"h": info["h"], "w0": info["w0"], "w1": info["w"][0]},
                    "l2": "inputs larger than L2 (2 x 256 MiB ping-pong buffers > 126 MB)"},
         "roofline": {"bound": "hbm", "achieved": achieved_gbs, "peak": peak, "unit": "GB/s",
-                     "frac": achieved_gbs / peak, "traffic": None, "peak_source": peak_src,
-                     "kernel": "fast2d phase kernel" if info["fast_kernel"] else "hybrid phase kernel",
+                     "frac": achieved_gbs / peak,
+                     "traffic": measured_traffic(cfg, {"h": info["h"], "w0": info["w0"]}),
+                     "traffic_source": "ncu dram__bytes_read.sum+dram__bytes_write.sum per launch "
+                                       f"(profiles/round1/traffic_{cfg}.json)",
+                     "alg_bytes_per_launch": alg_bytes_per_launch, "peak_source": peak_src,
+                     "kernel": KERNEL_NAMES[plan.executor_name],
                      "bytes_per_update": bpu, "avg_launch_ms": avg_launch_ms,
                      "tiled_hbm_roofline_gups": tiled_roof,
                      "kernel_share_of_step": prof["kernel_ms"] / args.steps / ms},

@@ -96,6 +96,14 @@ class Plan:
             out[name] = list(v) if isinstance(v, ctypes.Array) else v
         return out
 
+    @property
+    def executor_name(self) -> str:
+        """Which kernel family runs: fast2d / fdtd / fast3d (specialised) or generic / naive."""
+        i = self.info
+        if i["fast_kernel"]:
+            return "fdtd" if self.stencil.kind == "fdtd2d" else ("fast3d" if len(self.stencil.extents) == 3 else "fast2d")
+        return "naive" if i["executor"] == 2 else "generic"
+
     def launches(self) -> List[Dict[str, int]]:
         n = ctypes.c_int64()
         check(lib().stencil_plan_launches(self._h, None, 0, ctypes.byref(n)))
