@@ -72,27 +72,25 @@ struct FdtdArgs {
 cudaError_t launch_fdtd(int variant, const FdtdArgs& a, int grid, cudaStream_t s);
 size_t fdtd_smem_bytes(int dtype, int W);
 
-// 3D fast kernel.
-// 3D fast kernel (wavefront of smem-resident classical tiles, kernels/hex3d.cu).
+// 3D fast kernel (kernels/hex3d.cu): persistent CTAs run the classical tiles of every
+// hexagon of the launch as a tile-granular dependence wavefront, all levels of a tile in
+// shared memory.
 struct Fast3DArgs {
   void* buf[2];
   int64_t N0, N1, N2;
   int64_t tau0;
   int a_lo, a_hi, a_final;
   int64_t S0_lo, S0_hi, row_off;
-  int W, H, L, Q;          // box width, h, levels 2h+2, buffer planes (max rows + 2)
+  int W, H, L, Q;          // box width, h, levels 2h+2, buffer rows (max hexagon rows + 2)
   int64_t S1_lo, n1, S2_lo, n2;
   double k0, k1;
-  int* flags;
-  unsigned long long* counter;
-  long long* trace;  // optional (debug): per-item timestamps, see hex3d.cu
-  int dbg;           // debug timing modes (0 in production), see hex3d.cu
+  int* flags;                   // per tile completion flag, zeroed per launch
+  unsigned long long* counter;  // work counter, zeroed per launch
   int32_t lo[kMaxH], hi[kMaxH];
 };
-// Debug tracing of the 3D kernel (host-set device buffer; NULL disables).
-void fast3d_set_trace(long long* dev_buf, int64_t n_items_cap);
 cudaError_t launch_fast3d(int variant, const Fast3DArgs& a, int grid, cudaStream_t s);
-constexpr int kFast3DNY = 8, kFast3DNX = 32;  // classical tile of the 3D fast kernel
+constexpr int kFast3DNX = 32;            // classical tile width along x of the 3D fast kernel
+int fast3d_tile_lines(int dtype);        // classical tile height along y (32 fp32, 16 fp64)
 size_t fast3d_smem_bytes(int dtype, int Q);
 
 }  // namespace hexs

@@ -46,15 +46,15 @@ int fdtd_variant(int dtype, int h, int w0) {
   return dtype == 1 ? 1 : 0;
 }
 // 3D fast kernel: any (h, w0) whose two level buffers fit in shared memory
-// (2 * (w0 + 2h + 3) planes x 18 lines x 40 columns).
+// (2 x (w0 + 2h + 3) rows x (main + carry lines + carry columns) of one classical tile).
 int fast3d_variant(int kind, int dtype, int h, int w0) {
   if (kind != K_STAR3D7 && kind != K_GRADIENT3D && kind != K_BOX3D27) return -1;
   const int Q = w0 + 2 * h + 3;
   if (fast3d_smem_bytes(dtype, Q) > 200 * 1024 || 2 * h + 2 > kMaxH) return -1;
   return kind * 2 + dtype;
 }
-int fast3d_tile(int, int* wy, int* wx) {
-  *wy = kFast3DNY;
+int fast3d_tile(int variant, int* wy, int* wx) {
+  *wy = fast3d_tile_lines(variant & 1);
   *wx = kFast3DNX;
   return 0;
 }

@@ -261,14 +261,12 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
     p->w[q] = wq;
   }
 
-  // The 3D fast kernel moves whole 16-B groups with TMA, whose innermost box origin must be
-  // 16-B aligned: it skews the contiguous dimension by 4 per level (any integer skew >=
-  // delta1_i keeps eq. (14) valid, reading R16) and translates the x tiles by +1 (the
-  // translation offset of Sec. 4.2.3) so the inputs of a thread's four
-  // outputs start on a 16-B boundary.
+  // The 3D fast kernel moves whole 16-B groups (TMA boxes, vector loads/stores): it skews the
+  // contiguous dimension by 4 per level (any integer skew >= delta1_i keeps eq. (14) valid,
+  // reading R16), so every tile boundary of every level is 16-B aligned.
   if (ex == EXEC_FAST3D) {
     p->dcls[1] = std::max(p->dcls[1], 4);
-    p->ctrans[1] = 1;
+    p->ctrans[1] = 0;
   }
 
   // a3: launch table.  Order (T, 0), (T, 1), T ascending.
