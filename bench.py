@@ -168,6 +168,7 @@ def cpu_baseline(kind, ext, target_s=12.0):
     nthreads = oracle.max_threads()
     if kind == "fdtd2d":
         f = stencil_inputs.fields(ext, seed=0, n=3)
+        oracle.fdtd(*f, 1, nthreads=nthreads)  # warm-up (page faults, thread start)
         t0 = time.perf_counter()
         oracle.fdtd(*f, 2, nthreads=nthreads)
         dt = (time.perf_counter() - t0) / 2
@@ -178,6 +179,7 @@ def cpu_baseline(kind, ext, target_s=12.0):
         upd = ext[0] * ext[1] * steps
     else:
         g = stencil_inputs.uniform(ext, seed=0)
+        oracle.run(kind, g, 1, nthreads=nthreads)  # warm-up (page faults, thread start)
         t0 = time.perf_counter()
         oracle.run(kind, g, 2, nthreads=nthreads)
         dt = (time.perf_counter() - t0) / 2
@@ -253,9 +255,11 @@ def run_gpu(args, cfg):
     fields = make_inputs(kind, ext)
     st = Stencil(kind, ext)
     tile = {}
-    if args.tile:
-        h, w0 = (int(x) for x in args.tile.split(","))
-        tile = {"h": h, "w0": w0}
+    if args.tile:  # h,w0[,w1]: hexagon and (optionally) the first classical width
+        v = [int(x) for x in args.tile.split(",")]
+        tile = {"h": v[0], "w0": v[1]}
+        if len(v) > 2:
+            tile["w"] = (v[2], 0, 0)
     plan = Plan(st, T, **tile)
     info = plan.info
     host = [torch.from_numpy(f).pin_memory() for f in fields]
@@ -358,7 +362,7 @@ def main():
     ap.add_argument("--config", default="heat2d5", choices=sorted(CONFIGS))
     ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
     ap.add_argument("--no-cpu", action="store_true", help="skip the CPU oracle baseline")
-    ap.add_argument("--tile", default="", help="h,w0 override (tuning)")
+    ap.add_argument("--tile", default="", help="h,w0[,w1] override (tuning)")
     args = ap.parse_args()
     args.warmup = max(3, args.warmup)
     if args.impl == "reference":

@@ -45,6 +45,9 @@ def _deps_hash(paths):
     return h.hexdigest()[:16]
 
 
+EXTRA3D = []  # extra flags of the 3D kernel objects (debug builds)
+
+
 def _units():
     """(source, object, extra flags) for every translation unit."""
     headers = [os.path.join(dp, f) for dp, _, fs in os.walk(CSRC) for f in fs
@@ -52,10 +55,12 @@ def _units():
     units = []
     for src in ["desc.cpp", "plan.cpp"]:
         units.append((os.path.join(CSRC, src), "cxx", []))
-    for src in ["run.cu", "kernels/generic.cu", "kernels/registry.cu", "kernels/hex3d.cu", "kernels/fdtd.cu"]:
+    for src in ["run.cu", "kernels/generic.cu", "kernels/registry.cu", "kernels/fdtd.cu"]:
         units.append((os.path.join(CSRC, src), "nvcc", []))
     for vid in _variant_ids("fast2d_variants.h", "HEXS_FAST2D_VARIANTS"):
         units.append((os.path.join(KDIR, "fast2d_inst.cu"), "nvcc", [f"-DHEXS_VARIANT={vid}"]))
+    for vid in _variant_ids("fast3d_variants.h", "HEXS_FAST3D_VARIANTS"):
+        units.append((os.path.join(KDIR, "hex3d.cu"), "nvcc", [f"-DHEXS_F3_VARIANT={vid}"] + EXTRA3D))
     out = []
     for src, tool, extra in units:
         key = _deps_hash([src] + headers) + hashlib.sha1(" ".join(extra).encode()).hexdigest()[:8]
@@ -78,7 +83,8 @@ def _compile(unit, verbose=False):
     return obj, r.stderr
 
 
-def build_library(jobs: int = 0, verbose: bool = False) -> str:
+def build_library(jobs: int = 0, verbose: bool = False, lib: str = None) -> str:
+    LIB = lib or globals()["LIB"]
     os.makedirs(OBJ, exist_ok=True)
     os.makedirs(os.path.dirname(LIB), exist_ok=True)
     units = _units()
@@ -111,8 +117,13 @@ def main():
     ap = argparse.ArgumentParser()
     ap.add_argument("-j", type=int, default=0)
     ap.add_argument("-v", action="store_true")
+    ap.add_argument("--timing", action="store_true",
+                    help="also build lib/libhexstencil_tm.so with the 3D kernel's cycle accounting")
     args = ap.parse_args()
     print(build_library(args.j, args.v))
+    if args.timing:
+        EXTRA3D.append("-DHEXS_F3_TIMING")
+        print(build_library(args.j, args.v, lib=os.path.join(PKG, "lib", "libhexstencil_tm.so")))
     print(build_oracle())
 
 

@@ -9,7 +9,9 @@ import ctypes
 import os
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(_HERE, "lib", "libhexstencil.so")
+# HEXS_LIB selects an alternative build of the same library (e.g. the cycle-accounting
+# build of tools/f3_timing.py); the default is the in-tree product build.
+LIB_PATH = os.environ.get("HEXS_LIB") or os.path.join(_HERE, "lib", "libhexstencil.so")
 
 STATUS = {0: "STENCIL_OK", 1: "STENCIL_E_INVALID", 2: "STENCIL_E_UNSUPPORTED",
           3: "STENCIL_E_INFEASIBLE_TILE", 4: "STENCIL_E_OOM", 5: "STENCIL_E_CUDA",

@@ -63,6 +63,8 @@ struct Launch {
   int64_t row_off;
   // classical tile index ranges (generic executor)
   int64_t Slo[2], Shi[2];
+  // wavefront executors: first tile flag and work counter of this launch in the workspace
+  int64_t flag_first = 0, counter_idx = 0;
 };
 
 enum Executor { EXEC_GENERIC = 1, EXEC_NAIVE = 2, EXEC_FAST2D = 3, EXEC_FDTD = 4, EXEC_FAST3D = 5 };
@@ -110,7 +112,7 @@ stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* 
 int fast2d_variant(int kind, int dtype, int h, int w0);
 int fast2d_chunk_width(int variant);  // classical tile width w1 the kernel streams
 int fdtd_variant(int dtype, int h, int w0);
-int fast3d_variant(int kind, int dtype, int h, int w0);
+int fast3d_variant(int kind, int dtype, int h, int w0, int wy);
 int fast3d_tile(int variant, int* wy, int* wx);
 
 }  // namespace hexs

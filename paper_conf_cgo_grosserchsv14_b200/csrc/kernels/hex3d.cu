@@ -1,72 +1,97 @@
 // hex3d.cu -- the specialised sm_100a phase kernel for 3D single-field stencils of radius 1
 // (star3d7, gradient3d, box3d27) under the hybrid schedule: hexagonal over (t, z), classical
-// parallelogram tiles over y and x (eq. (14)).
+// parallelogram tiles over y and x (eq. (14)).  Compiled once per
+// (class, dtype, h, w0) of fast3d_variants.h (-DHEXS_F3_VARIANT=id).
 //
 // Mapping:
 //   * work item = one classical tile (S1, S2) of one hexagon S0 of the launch's (T, p): an
 //     NY x NX (y, x) parallelogram over the hexagon's 2h+2 levels and its rows z.  Skews: y
 //     by 1 per level (delta1_y = 1), x by 4 per level (any integer skew >= delta1_x keeps
 //     eq. (14) valid, reading R16) so every x-window this kernel moves is 16-B aligned;
+//   * the hexagon shape is a template parameter: every level's row range [lo(a), hi(a)] is a
+//     compile-time constant and each level's row sweep is fully unrolled (the paper's
+//     constraint-based unrolling); nothing in the sweep depends on the
+//     tile's position -- Dirichlet cells are repaired after the sweep in the few tiles that
+//     touch the domain edge, and stores carry a per-row predicate from a 32-bit row mask;
 //   * the tile keeps ALL its levels on chip: level a reads a shared-memory buffer holding
 //     level a-1 (rows x (NY+2) lines x (NX+5) columns) and writes the other buffer;
 //   * tile-granular dependences: the skew makes every dependence point to a tile with
 //     component-wise larger-or-equal (S1, S2), so a tile whose predecessors (S1-1, S2) and
 //     (S1, S2-1) have COMPLETED finds every value it reads, at every level, in global memory.
 //     Persistent CTAs take tiles in anti-diagonal order (S1 + S2, then S0, then S1), wait for
-//     the two predecessor flags once, and publish their own flag once (st.release.gpu) --
-//     no per-level cross-SM synchronisation;
+//     the two predecessor flags once, and publish their own flag once (st.release.gpu);
 //   * everything a tile reads from L2/HBM arrives by 3-D TMA tensor copies (SASS UTMALDG)
-//     completing on one mbarrier per buffer, one level ahead of the compute: the first level
-//     (issued during the previous tile's last level, which writes no shared memory), then
-//     per level the hexagon's In rows (its slanted-edge inputs) and the
-//     carries the predecessor tiles produced: 2 lines above and 5 columns left, staged into
-//     their own dense areas (a TMA box lands densely, so each area matches one box);
+//     completing on one mbarrier per buffer: the first level's whole buffer (issued during the
+//     previous tile's last level, which writes no shared memory), the In rows of every later
+//     level (the hexagon's slanted-edge inputs) two levels ahead, into rows
+//     the level in between neither reads nor writes, and per level the carries the
+//     predecessor tiles produced: 2 lines above and 5 columns left;
 //   * a thread owns one line and 4 consecutive x of the tile and sweeps z with a 3-row
 //     register window (z neighbours from registers, y neighbours from the level buffer, x
 //     edges by shuffle inside 8-lane groups);
 //   * results leave from registers: the Out rows (slanted upper edges and top row), every
-//     value of level T_steps, and the tile's last 2 lines / last 5 columns of every level
+//     value of level T_steps, and the tile's last 2 lines / last 2 quads of every level
 //     (its successors' carries) -- interleaved copy-out.
 #include <cuda.h>
 #include <cudaTypedefs.h>
 
 #include <cstdint>
 #include <type_traits>
+#include <utility>
 
 #include "../stencil_ops.cuh"
+#include "fast3d_variants.h"
 #include "launch.h"
 #include "tma.cuh"
+
+#ifndef HEXS_F3_VARIANT
+#error "hex3d.cu is compiled once per fast3d variant: -DHEXS_F3_VARIANT=<id>"
+#endif
 
 namespace hexs {
 namespace fast3d {
 
 constexpr int NX = kFast3DNX;  // tile columns (x)
+constexpr int NXP = NX + 4;    // shared-memory line pitch (spreads the per-line edge loads over banks)
 constexpr int NQ = NX / 4;     // column quads: one 8-lane group
 constexpr int SIGMA = 4;       // x skew per level
-template <typename T> constexpr int NY = sizeof(T) == 4 ? 32 : 16;  // tile lines (y)
-template <typename T> constexpr int NT = NY<T> * NQ;                 // threads: one per (line, quad)
 constexpr int CC = 8;          // carry-area columns (x = X0 - 4a - 4 .. X0 - 4a + 3)
 
-// Per buffer (level a's input = level a-1 values), Q rows (b = lo_min - 1 + r):
-//   main  [Q][NY][NX]     own region: y = Y0 - a + 1 + l, x = X0 - 4a + 4 + m
-//   lines [Q][2][NX]      carry lines: y = Y0 - a - 1 + l, x as main
-//   carry [Q][NY+2][CC]   carry columns: y = Y0 - a - 1 + l, x = X0 - 4a - 4 + c
-template <typename T> struct Lay {
-  static constexpr int MAIN = NY<T> * NX, LINES = 2 * NX, CARRY = (NY<T> + 2) * CC;
-  static constexpr int ROW = MAIN + LINES + CARRY;  // elements per row (all areas)
+// Hexagon of a radius-1 single-statement stencil (delta0 = delta1 = 1): rows b of level a
+// (SURVEY §8(a) closed form of eqs. (6)-(13)); buffer rows b = -1 .. 2h + w0 + 1.
+template <int H, int W0> struct Hex {
+  static constexpr int L = 2 * H + 2, Q = W0 + 2 * H + 3;
+  __host__ __device__ static constexpr int lo(int a) { return a <= H ? H - a : a - H - 1; }
+  __host__ __device__ static constexpr int hi(int a) { return a <= H ? H + W0 + a : 3 * H + 1 + W0 - a; }
+  // rows of level a that tiles of the next phase read (the slanted upper edges of the Out set)
+  __host__ __device__ static constexpr bool out_row(int a, int r) {
+    return a == H ? (r == lo(a) || r == hi(a)) : (a > H ? (r <= lo(a) + 1 || r >= hi(a) - 1) : false);
+  }
 };
-// one buffer, padded so the second one stays 128-B aligned (TMA destinations)
-template <typename T> __host__ __device__ constexpr size_t buf_elems(int Q) {
-  return ((size_t)Q * Lay<T>::ROW * sizeof(T) + 127) / 128 * 128 / sizeof(T);
-}
-template <typename T> constexpr size_t smem_bytes(int Q) { return 2 * buf_elems<T>(Q) * sizeof(T); }
+
+constexpr int al128(int bytes) { return (bytes + 127) / 128 * 128; }
+// One buffer (level a's input = level a-1 values), Q rows (buffer row rr = b + 1):
+//   main  [Q][NY][NXP]    own region: y = Y0 - a + 1 + l, x = X0 - 4a + 4 + m
+//   lines [Q][2][NXP]     carry lines: y = Y0 - a - 1 + l, x as main
+//   carry [Q][NY+2][CC]   carry columns: y = Y0 - a - 1 + l, x = X0 - 4a - 4 + c
+// Each area starts 128-B aligned (TMA destinations).  Offsets in elements.
+template <typename T, int Q, int NY> struct Lay {
+  static constexpr int MAIN = NY * NXP, LINES = 2 * NXP, CARRY = (NY + 2) * CC;
+  static constexpr int LINES_OFF = al128(Q * MAIN * (int)sizeof(T)) / (int)sizeof(T);
+  static constexpr int CARRY_OFF = al128((LINES_OFF + Q * LINES) * (int)sizeof(T)) / (int)sizeof(T);
+  static constexpr int BUF = al128((CARRY_OFF + Q * CARRY) * (int)sizeof(T)) / (int)sizeof(T);
+  static constexpr size_t SMEM = 2 * (size_t)BUF * sizeof(T);
+  static constexpr uint32_t FIRST_BYTES = (uint32_t)(Q * (MAIN + LINES + CARRY) * sizeof(T));
+  static constexpr uint32_t CARRY_BYTES = (uint32_t)(Q * (LINES + CARRY) * sizeof(T));
+  static constexpr uint32_t ROW_BYTES = (uint32_t)(MAIN * sizeof(T));
+};
 
 struct Maps {
-  CUtensorMap main[2];   // box {NX, NY, Q}
-  CUtensorMap lines[2];  // box {NX, 2, Q}
+  CUtensorMap main[2];   // box {NXP, NY, Q}
+  CUtensorMap lines[2];  // box {NXP, 2, Q}
   CUtensorMap carry[2];  // box {CC, NY+2, Q}
-  CUtensorMap in2[2];    // box {NX, NY, 2}
-  CUtensorMap in1[2];    // box {NX, NY, 1}
+  CUtensorMap in2[2];    // box {NXP, NY, 2}
+  CUtensorMap in1[2];    // box {NXP, NY, 1}
 };
 
 __device__ __forceinline__ int ld_acquire(const int* p) {
@@ -122,6 +147,9 @@ __device__ __forceinline__ double lds_if(bool pred, const double* p, double v) {
 // the column past the tile's quads).  Unused values are dead code.  Warp-uniform calls.
 template <typename T> struct Win { T v[3][6]; };
 
+// Two phases, so a row's shared-memory latency hides behind the previous rows' arithmetic:
+// load_win issues the loads (vector quads; the group's outer lanes also load their edge
+// column with a predicated scalar load), edges_win completes the edges by shuffle.
 template <typename T, bool ALL_EDGES>  // star / gradient stencils need the centre line's edges only
 __device__ __forceinline__ void load_win(Win<T>& w, const T* const (&p)[3], int q) {
 #pragma unroll
@@ -134,44 +162,105 @@ __device__ __forceinline__ void load_win(Win<T>& w, const T* const (&p)[3], int 
       const double2 u1 = reinterpret_cast<const double2*>(p[l])[1];
       w.v[l][1] = u0.x; w.v[l][2] = u0.y; w.v[l][3] = u1.x; w.v[l][4] = u1.y;
     }
-    // interior edges by shuffle; the group's outer lanes load theirs with a predicated
-    // LDS (no branch, so the warp never diverges around the shuffles)
     if (ALL_EDGES || l == 1) {
-      w.v[l][0] = lds_if(q == 0, p[l] - 1, __shfl_up_sync(0xffffffffu, w.v[l][4], 1, NQ));
-      w.v[l][5] = lds_if(q == NQ - 1, p[l] + 4, __shfl_down_sync(0xffffffffu, w.v[l][1], 1, NQ));
+      w.v[l][0] = lds_if(q == 0, p[l] - 1, T(0));
+      w.v[l][5] = lds_if(q == NQ - 1, p[l] + 4, T(0));
     } else {
       w.v[l][0] = w.v[l][5] = T(0);  // never used by this stencil
     }
   }
 }
+template <typename T, bool ALL_EDGES>
+__device__ __forceinline__ void edges_win(Win<T>& w, int q) {
+#pragma unroll
+  for (int l = 0; l < 3; ++l) {
+    if (ALL_EDGES || l == 1) {
+      const T lft = __shfl_up_sync(0xffffffffu, w.v[l][4], 1, NQ);
+      const T rgt = __shfl_down_sync(0xffffffffu, w.v[l][1], 1, NQ);
+      w.v[l][0] = q != 0 ? lft : w.v[l][0];
+      w.v[l][5] = q != NQ - 1 ? rgt : w.v[l][5];
+    }
+  }
+}
 
-template <typename T, int KIND>
-__global__ void __launch_bounds__(NT<T>, 1) fast3d_kernel(const __grid_constant__ Fast3DArgs g,
-                                                          const __grid_constant__ Maps mp) {
-  constexpr int LNY = NY<T>;
-  using LY = Lay<T>;
+// Optional per-CTA cycle accounting (debug builds: -DHEXS_F3_TIMING): thread 0 (the TMA
+// issuer) and thread 64 (a compute-only warp) add the cycles spent per category.
+#ifdef HEXS_F3_TIMING
+__device__ unsigned long long g_f3_tm[1024][2][8];
+#define F3_TM_DECL long long tm_t = clock64();
+#define F3_TM(k)                                                                     \
+  do {                                                                               \
+    if (threadIdx.x == NC || threadIdx.x == 64) {                                    \
+      const long long now = clock64();                                               \
+      atomicAdd(&g_f3_tm[blockIdx.x][threadIdx.x == NC ? 0 : 1][k], (unsigned long long)(now - tm_t)); \
+      tm_t = now;                                                                    \
+    }                                                                                \
+  } while (0)
+#else
+#define F3_TM_DECL
+#define F3_TM(k) \
+  do {           \
+  } while (0)
+#endif
+
+__device__ __forceinline__ void named_barrier_sync(int id, int nthreads) {
+  asm volatile("bar.sync %0, %1;" ::"r"(id), "r"(nthreads) : "memory");
+}
+
+template <int... As, typename F>
+__device__ __forceinline__ void for_levels(F&& f, std::integer_sequence<int, As...>) {
+  (f(std::integral_constant<int, As>{}), ...);
+}
+
+// NY tile lines (y); ZS threads per (line, quad), each sweeping 1/ZS of a level's rows;
+// MINB CTAs per SM; plus one producer warp
+template <typename T, int KIND, int H, int W0, int NY, int MINB, int ZS>
+__global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const __grid_constant__ Fast3DArgs g,
+                                                                   const __grid_constant__ Maps mp) {
+  using HX = Hex<H, W0>;
+  constexpr int LNY = NY, Q = HX::Q, L = HX::L;
+  using LY = Lay<T, Q, NY>;
   extern __shared__ __align__(1024) unsigned char smem_raw[];  // dynamic base: 1024-B aligned
   T* const sbase = reinterpret_cast<T*>(smem_raw);  // stays a shared-space pointer (LDS/STS)
-  __shared__ __align__(8) uint64_t full[2];
-  __shared__ long long item_s[2][3];  // [current, next] (S0, q1, q2); S0 < 0: none
+  constexpr int NC = ZS * NY * NQ, NCW = NC / 32;  // compute threads / warps; warp NCW produces
+  __shared__ __align__(8) uint64_t full[2];   // buffer filled (producer arrival + TMA bytes)
+  __shared__ __align__(8) uint64_t empty[2];  // buffer consumed (one arrival per compute warp)
+  __shared__ long long item_s[2][3];          // tile ring (S0, q1, q2); S0 < 0: no more work
   const int tid = threadIdx.x;
-  const int ly = tid / NQ, q = tid % NQ;  // line, column quad
-  const int Q = g.Q;
+  const int zpart = tid / (NY * NQ);                             // row part (< ZS; producer: ZS)
+  const int ly = (tid % (NY * NQ)) / NQ, q = tid % NQ;           // line, column quad
   const int64_t n1 = g.n1, n2 = g.n2, ns0 = g.S0_hi - g.S0_lo + 1, n_items = ns0 * n1 * n2;
   const int64_t N0 = g.N0, N1 = g.N1, N2 = g.N2, plane = N1 * N2;
-  int lo_min = 1 << 30;
-  for (int a = 0; a < g.L; ++a) lo_min = min(lo_min, (int)g.lo[a]);
-  const int zoff = lo_min - 1;  // b of buffer row 0
-  const int BE = (int)buf_elems<T>(Q);
-  auto main_of = [&](int b) { return sbase + b * BE; };
-  auto lines_of = [&](int b) { return sbase + b * BE + Q * LY::MAIN; };
-  auto carry_of = [&](int b) { return sbase + b * BE + Q * (LY::MAIN + LY::LINES); };
+  const int a_lo = g.a_lo, a_hi = g.a_hi;
+
+  // per-thread window lines k = 0..2 (input-frame line ly + k): element offset in a buffer
+  // at buffer row 0, and the row pitch of the area they live in
+  int woff[3], wpitch[3];
+#pragma unroll
+  for (int k = 0; k < 3; ++k) {
+    const int l = ly + k;
+    if (q == 0) {
+      woff[k] = LY::CARRY_OFF + l * CC + 4;
+      wpitch[k] = LY::CARRY;
+    } else if (l < 2) {
+      woff[k] = LY::LINES_OFF + l * NXP + 4 * q - 4;
+      wpitch[k] = LY::LINES;
+    } else {
+      woff[k] = (l - 2) * NXP + 4 * q - 4;
+      wpitch[k] = LY::MAIN;
+    }
+  }
+  const int sts_off = ly * NXP + 4 * q;                  // + row * MAIN in the output buffer
+  const bool cthr = (ly >= LNY - 2) || (q >= NQ - 2);   // writes its successors' carries
 
   if (tid == 0) {
     mbar_init(&full[0], 1);
     mbar_init(&full[1], 1);
+    mbar_init(&empty[0], NCW);
+    mbar_init(&empty[1], NCW);
     mbar_fence_init();
   }
+  __syncthreads();
   // decode the anti-diagonal order: d = q1 + q2 (outer), then S0, then q1
   auto decode = [&](int64_t it, long long* o) {
     o[0] = -1;
@@ -196,212 +285,294 @@ __global__ void __launch_bounds__(NT<T>, 1) fast3d_kernel(const __grid_constant_
     Y0 = (int)((g.S1_lo + it[1]) * LNY);
     X0 = (int)((g.S2_lo + it[2]) * NX);
   };
-  // Level a's input buffer a & 1 for a tile: the parts that come from global memory (all of
-  // it for the first level, else carry lines / columns + In rows).  Thread 0 only.
-  auto issue_level = [&](const long long* it, int a, bool first) {
+  auto buf_of = [&](int b) { return sbase + b * LY::BUF; };
+  // ---- TMA issue (thread 0 only) ----
+  // the whole input buffer of level a (first level of a tile): no dependence on predecessors
+  auto issue_first = [&](const long long* it, int a) {
     int64_t i0;
     int X0, Y0;
     tile_origin(it, i0, X0, Y0);
     const int b = a & 1, par = (int)((g.tau0 + a) & 1);
-    const int z0 = (int)(i0 + zoff);
+    const int z0 = (int)(i0 - 1), xo = X0 - SIGMA * a, yo = Y0 - a;
+    T* B = buf_of(b);
+    mbar_arrive_expect_tx(&full[b], LY::FIRST_BYTES);
+    tma_3d(B, &mp.main[par], xo + 4, yo + 1, z0, &full[b]);
+    tma_3d(B + LY::LINES_OFF, &mp.lines[par], xo + 4, yo - 1, z0, &full[b]);
+    tma_3d(B + LY::CARRY_OFF, &mp.carry[par], xo - 4, yo - 1, z0, &full[b]);
+  };
+  // In rows of level a: buffer rows level a reads ([lo(a)-1, hi(a)+1]) that level a-1 does
+  // not compute (0, 1 or 2 per side)
+  auto in_rows = [&](int a, int* lo2, int* n2_) {
+    const int need_lo = HX::lo(a) - 1, need_hi = HX::hi(a) + 1, clo = HX::lo(a - 1), chi = HX::hi(a - 1);
+    lo2[0] = need_lo; n2_[0] = need_lo < clo ? clo - need_lo : 0;
+    lo2[1] = chi + 1; n2_[1] = need_hi > chi ? need_hi - chi : 0;
+  };
+  auto issue_in = [&](const long long* it, int a) {
+    int64_t i0;
+    int X0, Y0;
+    tile_origin(it, i0, X0, Y0);
+    const int b = a & 1, par = (int)((g.tau0 + a) & 1);
     const int xo = X0 - SIGMA * a, yo = Y0 - a;
-    uint32_t elems = (uint32_t)(Q * (LY::LINES + LY::CARRY));
-    // In rows of level a: buffer rows level a reads ([lo(a)-1, hi(a)+1]) that level a-1
-    // does not compute
-    int in_lo[2] = {0, 0}, in_n[2] = {0, 0};
-    if (first) {
-      elems += (uint32_t)(Q * LY::MAIN);
-    } else {
-      const int need_lo = g.lo[a] - 1, need_hi = g.hi[a] + 1, clo = g.lo[a - 1], chi = g.hi[a - 1];
-      if (need_lo < clo) in_lo[0] = need_lo, in_n[0] = clo - need_lo;
-      if (need_hi > chi) in_lo[1] = chi + 1, in_n[1] = need_hi - chi;
-      elems += (uint32_t)((in_n[0] + in_n[1]) * LY::MAIN);
-    }
-    fence_proxy_async_smem();  // earlier generic accesses of this buffer before TMA writes
-    mbar_arrive_expect_tx(&full[b], elems * (uint32_t)sizeof(T));
-    tma_3d(lines_of(b), &mp.lines[par], xo + 4, yo - 1, z0, &full[b]);
-    tma_3d(carry_of(b), &mp.carry[par], xo - 4, yo - 1, z0, &full[b]);
-    if (first) {
-      tma_3d(main_of(b), &mp.main[par], xo + 4, yo + 1, z0, &full[b]);
-    } else {
-      for (int s = 0; s < 2; ++s) {
-        for (int k = 0; k < in_n[s];) {  // In rows: boxes of 2 rows, then 1
-          const int bb = in_lo[s] + k;
-          T* dst = main_of(b) + (size_t)(bb - zoff) * LY::MAIN;
-          if (in_n[s] - k >= 2) {
-            tma_3d(dst, &mp.in2[par], xo + 4, yo + 1, (int)(i0 + bb), &full[b]);
-            k += 2;
-          } else {
-            tma_3d(dst, &mp.in1[par], xo + 4, yo + 1, (int)(i0 + bb), &full[b]);
-            k += 1;
-          }
+    int lo2[2], nn[2];
+    in_rows(a, lo2, nn);
+    for (int s = 0; s < 2; ++s)
+      for (int k = 0; k < nn[s];) {
+        const int bb = lo2[s] + k;
+        T* dst = buf_of(b) + (bb + 1) * LY::MAIN;
+        if (nn[s] - k >= 2) {
+          tma_3d(dst, &mp.in2[par], xo + 4, yo + 1, (int)(i0 + bb), &full[b]);
+          k += 2;
+        } else {
+          tma_3d(dst, &mp.in1[par], xo + 4, yo + 1, (int)(i0 + bb), &full[b]);
+          k += 1;
         }
       }
-    }
+  };
+  auto in_bytes = [&](int a) {
+    int lo2[2], nn[2];
+    in_rows(a, lo2, nn);
+    return (uint32_t)(nn[0] + nn[1]) * LY::ROW_BYTES;
+  };
+  auto issue_carries = [&](const long long* it, int a) {
+    int64_t i0;
+    int X0, Y0;
+    tile_origin(it, i0, X0, Y0);
+    const int b = a & 1, par = (int)((g.tau0 + a) & 1);
+    const int z0 = (int)(i0 - 1), xo = X0 - SIGMA * a, yo = Y0 - a;
+    tma_3d(buf_of(b) + LY::LINES_OFF, &mp.lines[par], xo + 4, yo - 1, z0, &full[b]);
+    tma_3d(buf_of(b) + LY::CARRY_OFF, &mp.carry[par], xo - 4, yo - 1, z0, &full[b]);
   };
 
+  F3_TM_DECL
+  if (tid >= NC) {
+    // ================= producer warp (one lane): tiles, predecessor flags, TMA =================
+    // Fill k of a buffer waits for the level that consumed fill k-1 (empty[b] completion
+    // k-1); fill(a_lo) = the whole first-level buffer, fill(a) = the In rows of level a and
+    // the carries its predecessors produced at level a-1 (they are complete before
+    // fill(a_lo + 1) is issued).
+    if (tid == NC) {
+      uint32_t fills[2] = {0u, 0u};
+      int slot = 0;
+      while (true) {
+        long long* it = item_s[slot];
+        decode((int64_t)atomicAdd(g.counter, 1ull), it);
+        if (it[0] < 0) {  // no more tiles: wake the compute warps with an empty fill
+          const int b0 = a_lo & 1;
+          if (fills[b0] > 0) mbar_wait_parity(&empty[b0], (fills[b0] - 1) & 1u);
+          mbar_arrive(&full[b0]);
+          break;
+        }
+        const int64_t base = (it[0] - g.S0_lo) * n1 * n2;
+        for (int a = a_lo; a <= a_hi; ++a) {
+          const int b = a & 1;
+          if (fills[b] > 0) mbar_wait_parity(&empty[b], (fills[b] - 1) & 1u);
+          F3_TM(0);
+          fence_proxy_async_smem();
+          if (a == a_lo) {
+            issue_first(it, a);
+          } else {
+            if (a == a_lo + 1) {  // predecessors complete: their carries are in global memory
+              const int* f = g.flags + base;
+              if (it[1] > 0)
+                while (ld_acquire(f + (it[1] - 1) * n2 + it[2]) == 0) __nanosleep(64);
+              if (it[2] > 0)
+                while (ld_acquire(f + it[1] * n2 + it[2] - 1) == 0) __nanosleep(64);
+              fence_proxy_async_global();
+              F3_TM(2);
+            }
+            mbar_arrive_expect_tx(&full[b], LY::CARRY_BYTES + (a <= H + 1 ? in_bytes(a) : 0u));
+            if (a <= H + 1) issue_in(it, a);
+            issue_carries(it, a);
+          }
+          ++fills[b];
+          F3_TM(4);
+        }
+        slot ^= 1;
+      }
+    }
+    return;
+  }
+
+  // ================= compute warps =================
   uint32_t ph = 0u;  // parity bit per buffer
   const Coef<T> cf{(T)g.k0, (T)g.k1};
-  // the next tile's first level can be staged during this tile's last level (which writes
-  // no shared memory) when that buffer is the other one: a_hi - a_lo odd
-  const bool early = ((g.a_hi - g.a_lo) & 1) != 0;
-  if (tid == 0) {
-    decode((int64_t)atomicAdd(g.counter, 1ull), item_s[0]);
-    if (item_s[0][0] >= 0) issue_level(item_s[0], g.a_lo, true);
-  }
-  __syncthreads();
-  int cur = 0;
+  const int lane = tid & 31;
+  int slot = 0;
   while (true) {
-    const long long* it = item_s[cur];
+    {
+      const int b0 = a_lo & 1;  // the tile's first fill publishes its item
+      mbar_wait_parity(&full[b0], (ph >> b0) & 1u);
+    }
+    const long long* it = item_s[slot];
     if (it[0] < 0) break;
     int64_t i0;
     int X0, Y0;
     tile_origin(it, i0, X0, Y0);
     const int64_t base = (it[0] - g.S0_lo) * n1 * n2;
     int* const my_flag = g.flags + base + it[1] * n2 + it[2];
-    bool deps_ok = false;
-    for (int a = g.a_lo; a <= g.a_hi; ++a) {
-      const int b = a & 1, nb = b ^ 1;
-      mbar_wait_parity(&full[b], (ph >> b) & 1u);
-      ph ^= 1u << b;
-      __syncthreads();  // level a-1's buffer writes visible; buffer nb no longer read
-      if (tid == 0) {
-        if (a < g.a_hi) {
-          if (!deps_ok) {  // predecessors complete: their carries are in global memory
-            if (it[1] > 0)
-              while (ld_acquire(g.flags + base + (it[1] - 1) * n2 + it[2]) == 0) __nanosleep(32);
-            if (it[2] > 0)
-              while (ld_acquire(g.flags + base + it[1] * n2 + it[2] - 1) == 0) __nanosleep(32);
-            fence_proxy_async_global();
-            deps_ok = true;
-          }
-          issue_level(it, a + 1, false);
-        } else {
-          decode((int64_t)atomicAdd(g.counter, 1ull), item_s[cur ^ 1]);
-          if (early && item_s[cur ^ 1][0] >= 0) issue_level(item_s[cur ^ 1], g.a_lo, true);
-        }
-      }
+    // rows b of the hexagon whose z is an interior point (bit b); Dirichlet rows excluded
+    uint32_t zmask = 0u;
+#pragma unroll
+    for (int b = 0; b <= 2 * H + W0; ++b) zmask |= (i0 + b >= 1 && i0 + b <= N0 - 2 ? 1u : 0u) << b;
+    // a tile that never touches a domain edge needs no repair pass
+    const bool edge = zmask != (2u << (2 * H + W0)) - 1u || Y0 - a_hi < 1 || Y0 - a_lo + LNY - 1 > N1 - 2 ||
+                      X0 - SIGMA * a_hi < 1 || X0 - SIGMA * a_lo + NX - 1 > N2 - 2;
+    F3_TM(3);
 
-      // ---- compute level a: line y = Y0 - a + ly, x = X0 - 4a + 4q + j, rows [lo, hi]
-      const int rlo = g.lo[a], rhi = g.hi[a];
-      const int y = Y0 - a + ly;
-      const int xb = X0 - SIGMA * a + 4 * q;
-      const bool to_smem = a < g.a_hi;
-      // window line pointers (input-frame line l = ly + k) at buffer row rlo - 1
-      const T* P[3];
-      int pitch[3];
-#pragma unroll
-      for (int k = 0; k < 3; ++k) {
-        const int l = ly + k, r = rlo - 1 - zoff;
-        if (q == 0) {
-          P[k] = carry_of(b) + ((size_t)r * (LNY + 2) + l) * CC + 4;
-          pitch[k] = (LNY + 2) * CC;
-        } else if (l < 2) {
-          P[k] = lines_of(b) + ((size_t)r * 2 + l) * NX + 4 * q - 4;
-          pitch[k] = 2 * NX;
-        } else {
-          P[k] = main_of(b) + ((size_t)r * LNY + l - 2) * NX + 4 * q - 4;
-          pitch[k] = LY::MAIN;
-        }
-      }
-      T* const Wn = main_of(nb) + ((size_t)(rlo - zoff) * LNY + ly) * NX + 4 * q;  // row rlo of level a
-      // per-output masks: interior in (y, x); successors' carries (last 2 lines, last 5 cols)
-      uint32_t vmask = 0u;
-#pragma unroll
-      for (int j = 0; j < 4; ++j)
-        vmask |= (y >= 1 && y <= N1 - 2 && xb + j >= 1 && xb + j <= N2 - 2 ? 1u : 0u) << j;
-      const uint32_t cstatic = (ly >= LNY - 2) ? 0xFu : (q == NQ - 1 ? 0xFu : (q == NQ - 2 ? 0x8u : 0u));
-      const uint32_t cmask = to_smem ? (vmask & cstatic) : 0u;
-      int flo = -(1 << 30), fhi = 1 << 30;  // rows stored in full: r <= flo or r >= fhi
-      if (a == g.a_final || a == g.L - 1) flo = 1 << 30, fhi = -(1 << 30);
-      else if (a == g.H) flo = rlo, fhi = rhi;
-      else if (a > g.H) flo = rlo + 1, fhi = rhi - 1;
-      T* gp = static_cast<T*>(g.buf[(g.tau0 + a + 1) & 1]) + (i0 + rlo) * plane + (int64_t)y * N2 + xb;
-      const bool fast = __all_sync(0xffffffffu, vmask == 0xFu && i0 + rlo >= 1 && i0 + rhi <= N0 - 2);
+    for_levels(
+        [&](auto ac) {
+          constexpr int A = decltype(ac)::value;
+          if (A < a_lo || A > a_hi) return;
+          constexpr int b = A & 1, nb = b ^ 1;
+          constexpr int LO = HX::lo(A), HI = HX::hi(A);
+          // this thread's rows: N consecutive rows from R0 (the parts of an odd row count
+          // share one row, computed twice with identical results)
+          constexpr int N = (HI - LO + 1 + ZS - 1) / ZS;
+          const int R0 = zpart == 0 ? LO : HI - N + 1;
+          const int dR = R0 - LO;
+          if (A != a_lo) mbar_wait_parity(&full[b], (ph >> b) & 1u);
+          ph ^= 1u << b;
+          F3_TM(0);
+          named_barrier_sync(1, NC);  // level A-1's buffer writes visible to every compute warp
+          F3_TM(1);
 
-      auto sweep = [&](auto fast_c) {
-        constexpr bool FAST = decltype(fast_c)::value;
-        auto step = [&](int r, const Win<T>& Wp, const Win<T>& Wc, const Win<T>& Wx) {
-          uint32_t okm = vmask;
-          if constexpr (!FAST) {
-            const int64_t z = i0 + r;
-            if (z < 1 || z > N0 - 2) okm = 0u;
-          }
-          T out[4];
+          // ---- compute level A: line y = Y0 - A + ly, x = X0 - 4A + 4q + j, rows [LO, HI]
+          const T* const B = buf_of(b);
+          const T* P[3];
 #pragma unroll
-          for (int j = 0; j < 4; ++j) {
-            T x[3][3][3];
+          for (int k = 0; k < 3; ++k) P[k] = B + woff[k] + R0 * wpitch[k];  // window row R0 - 1
+          T* const Wn = buf_of(nb) + (R0 + 1) * LY::MAIN + sts_off;          // output row R0
+          const int y = Y0 - A + ly;
+          const int xb = X0 - SIGMA * A + 4 * q;
+          const bool to_smem = A < a_hi;
+          // whole-quad store validity (y interior, quad inside [0, N2)); the Dirichlet columns
+          // x = 0 and x = N2-1 inside a valid quad keep their value by a select
+          const bool vq = y >= 1 && y <= N1 - 2 && xb >= 0 && xb + 3 <= N2 - 1;
+          const bool xl = xb == 0, xr = xb + 3 == N2 - 1;
+          const bool st_all = A == g.a_final || A == L - 1;
+          const uint32_t zm_out = vq ? zmask : 0u;
+          const uint32_t zm_non = (vq && (st_all || (cthr && to_smem))) ? zmask : 0u;
+          // per-row store predicate, bit i = row R0 + i (Out rows: slanted upper edges)
+          constexpr uint32_t OMASK = [] {
+            uint32_t m = 0u;
+            for (int r = 0; r < 32; ++r) m |= (HX::out_row(A, r) ? 1u : 0u) << r;
+            return m;
+          }();
+          const uint32_t zsel = ((OMASK & zm_out) | (~OMASK & zm_non)) >> R0;
+          // store pointer of row LO, advanced one plane per row (a predicated store per row)
+          T* gp = static_cast<T*>(g.buf[(g.tau0 + A + 1) & 1]) + (i0 + R0) * plane + (int64_t)y * N2 + xb;
+
+          const T* Pr[3] = {P[0], P[1], P[2]};
+          auto adv = [&]() {
 #pragma unroll
-            for (int dy = 0; dy < 3; ++dy)
+            for (int k = 0; k < 3; ++k) Pr[k] += wpitch[k];
+          };
+          constexpr bool E27 = KIND == K_BOX3D27;
+          // one output row i from the windows of rows i-1, i, i+1 (registers)
+          auto step = [&](int i, const Win<T>& wm, const Win<T>& wc, const Win<T>& wp) {
+            T out[4];
 #pragma unroll
-              for (int dx = 0; dx < 3; ++dx) {
-                x[0][dy][dx] = Wp.v[dy][j + dx];
-                x[1][dy][dx] = Wc.v[dy][j + dx];
-                x[2][dy][dx] = Wx.v[dy][j + dx];
+            for (int j = 0; j < 4; ++j) {
+              T x[3][3][3];
+#pragma unroll
+              for (int dy = 0; dy < 3; ++dy)
+#pragma unroll
+                for (int dx = 0; dx < 3; ++dx) {
+                  x[0][dy][dx] = wm.v[dy][j + dx];
+                  x[1][dy][dx] = wc.v[dy][j + dx];
+                  x[2][dy][dx] = wp.v[dy][j + dx];
+                }
+              out[j] = apply<T, KIND>(x, cf);
+            }
+            out[0] = xl ? wc.v[1][1] : out[0];
+            out[3] = xr ? wc.v[1][4] : out[3];
+            if (to_smem) {
+              T* p = Wn + i * LY::MAIN;
+              if constexpr (sizeof(T) == 4) {
+                reinterpret_cast<float4*>(p)[0] = make_float4(out[0], out[1], out[2], out[3]);
+              } else {
+                reinterpret_cast<double2*>(p)[0] = make_double2(out[0], out[1]);
+                reinterpret_cast<double2*>(p)[1] = make_double2(out[2], out[3]);
               }
-            const T v = apply<T, KIND>(x, cf);
-            if constexpr (FAST) out[j] = v;
-            else out[j] = ((okm >> j) & 1u) ? v : x[1][1][1];
-          }
-          if (to_smem) {
-            T* p = Wn + (size_t)(r - rlo) * LY::MAIN;
-            if constexpr (sizeof(T) == 4) {
-              reinterpret_cast<float4*>(p)[0] = make_float4(out[0], out[1], out[2], out[3]);
-            } else {
-              reinterpret_cast<double2*>(p)[0] = make_double2(out[0], out[1]);
-              reinterpret_cast<double2*>(p)[1] = make_double2(out[2], out[3]);
+            }
+            if ((zsel >> i) & 1u) {
+              if constexpr (sizeof(T) == 4) {
+                reinterpret_cast<float4*>(gp)[0] = make_float4(out[0], out[1], out[2], out[3]);
+              } else {
+                reinterpret_cast<double2*>(gp)[0] = make_double2(out[0], out[1]);
+                reinterpret_cast<double2*>(gp)[1] = make_double2(out[2], out[3]);
+              }
+            }
+            gp += plane;
+          };
+          if constexpr (KIND == K_STAR3D7) {
+            // short per-point expression: the whole sweep unrolled and software-pipelined
+            // (loads of row i+3, edges of row i+2, arithmetic of row i+1)
+            Win<T> w[N + 2];
+            load_win<T, E27>(w[0], Pr, q);
+            adv();
+            load_win<T, E27>(w[1], Pr, q);
+            adv();
+            edges_win<T, E27>(w[0], q);
+            load_win<T, E27>(w[2], Pr, q);
+            adv();
+            edges_win<T, E27>(w[1], q);
+#pragma unroll
+            for (int i = 0; i < N; ++i) {
+              if (i + 3 < N + 2) {
+                load_win<T, E27>(w[i + 3], Pr, q);
+                adv();
+              }
+              edges_win<T, E27>(w[i + 2], q);
+              step(i, w[i], w[i + 1], w[i + 2]);
+            }
+          } else {
+            // long per-point expressions (IEEE sqrt / div, 27 operands): a rolled sweep with a
+            // 3-row register window keeps the level's code small enough for the i-cache
+            Win<T> wa, wb, wc;
+            auto ld = [&](Win<T>& w) {
+              load_win<T, E27>(w, Pr, q);
+              adv();
+              edges_win<T, E27>(w, q);
+            };
+            ld(wa);
+            ld(wb);
+#pragma unroll 1
+            for (int i = 0; i < N; i += 3) {
+              ld(wc);
+              step(i, wa, wb, wc);
+              if (i + 1 >= N) break;
+              ld(wa);
+              step(i + 1, wb, wc, wa);
+              if (i + 2 >= N) break;
+              ld(wb);
+              step(i + 2, wc, wa, wb);
             }
           }
-          const uint32_t sm_ = (r <= flo || r >= fhi) ? okm : (okm & cmask);
-          if (sm_ == 0xFu) {
-            if constexpr (sizeof(T) == 4) {
-              reinterpret_cast<float4*>(gp)[0] = make_float4(out[0], out[1], out[2], out[3]);
-            } else {
-              reinterpret_cast<double2*>(gp)[0] = make_double2(out[0], out[1]);
-              reinterpret_cast<double2*>(gp)[1] = make_double2(out[2], out[3]);
+          // ---- Dirichlet repair (domain-edge tiles): cells on the boundary lines / rows keep
+          // their value in the level buffer; it is the centre of their own stencil window
+          if (edge && to_smem) {
+            const bool yb = y == 0 || y == N1 - 1;
+            for (int r = R0; r < R0 + N; ++r) {
+              if (yb || !((zmask >> r) & 1u)) {
+                const T* c = P[1] + (r - R0 + 1) * wpitch[1];
+                T* o = Wn + (r - R0) * LY::MAIN;
+#pragma unroll
+                for (int j = 0; j < 4; ++j) o[j] = c[j];
+              }
             }
-          } else if (sm_) {
-#pragma unroll
-            for (int j = 0; j < 4; ++j)
-              if ((sm_ >> j) & 1u) gp[j] = out[j];
           }
-          gp += plane;
-        };
-        const T* Pr[3] = {P[0], P[1], P[2]};
-        auto adv = [&]() {
-#pragma unroll
-          for (int k = 0; k < 3; ++k) Pr[k] += pitch[k];
-        };
-        Win<T> wa, wb, wc;
-        load_win<T, KIND == K_BOX3D27>(wa, Pr, q);  // row rlo - 1
-        adv();
-        load_win<T, KIND == K_BOX3D27>(wb, Pr, q);  // row rlo
-        adv();
-        int r = rlo;
-        while (true) {
-          load_win<T, KIND == K_BOX3D27>(wc, Pr, q);
-          adv();
-          step(r, wa, wb, wc);
-          if (++r > rhi) break;
-          load_win<T, KIND == K_BOX3D27>(wa, Pr, q);
-          adv();
-          step(r, wb, wc, wa);
-          if (++r > rhi) break;
-          load_win<T, KIND == K_BOX3D27>(wb, Pr, q);
-          adv();
-          step(r, wc, wa, wb);
-          if (++r > rhi) break;
-        }
-      };
-      if (fast) sweep(std::true_type{});
-      else sweep(std::false_type{});
-    }
-    __syncthreads();  // the tile's stores are issued by every thread; item_s[cur^1] visible
-    if (tid == 0) {
-      st_release(my_flag, 1);
-      if (!early && item_s[cur ^ 1][0] >= 0) issue_level(item_s[cur ^ 1], g.a_lo, true);
-    }
-    cur ^= 1;
+          // buffer b consumed (and this warp's generic writes of nb ordered before later TMA)
+          fence_proxy_async_smem();
+          __syncwarp();
+          if (lane == 0) mbar_arrive(&empty[b]);
+          F3_TM(3);
+        },
+        std::make_integer_sequence<int, L>{});
+    named_barrier_sync(1, NC);  // every compute thread's stores of the tile are issued
+    F3_TM(1);
+    if (tid == 0) st_release(my_flag, 1);
+    slot ^= 1;
   }
 }
 
@@ -430,56 +601,67 @@ static bool encode(CUtensorMap* map, void* base, const Fast3DArgs& a, uint32_t b
             CU_TENSOR_MAP_L2_PROMOTION_L2_128B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE) == CUDA_SUCCESS;
 }
 
-template <typename T, int KIND>
+template <typename T, int KIND, int H, int W0, int NY, int MINB, int ZS>
 cudaError_t launch_t(const Fast3DArgs& a, cudaStream_t s) {
+  using LY = Lay<T, Hex<H, W0>::Q, NY>;
+  constexpr int NT = ZS * NY * NQ + 32;  // compute threads + the producer warp
   static int grid = 0;
-  static size_t attr_bytes = 0;
-  const size_t smem = smem_bytes<T>(a.Q);
-  if (smem > attr_bytes) {
-    cudaError_t e = cudaFuncSetAttribute(fast3d_kernel<T, KIND>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-    if (e != cudaSuccess) return e;
-    attr_bytes = smem;
-    grid = 0;
-  }
+  constexpr size_t smem = LY::SMEM;
+  auto kern = fast3d_kernel<T, KIND, H, W0, NY, MINB, ZS>;
   if (grid == 0) {
+    cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+    if (e != cudaSuccess) return e;
     int dev = 0, sms = 0, per_sm = 0;
     cudaGetDevice(&dev);
     cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
-    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, fast3d_kernel<T, KIND>, NT<T>, smem);
+    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, NT, smem);
     grid = sms * (per_sm > 0 ? per_sm : 1);
   }
+  if (a.Q != Hex<H, W0>::Q || a.L != Hex<H, W0>::L) return cudaErrorInvalidValue;
   Maps m;
-  const uint32_t Q = (uint32_t)a.Q, ny = (uint32_t)NY<T>;
+  const uint32_t Q = (uint32_t)a.Q, ny = (uint32_t)NY;
   for (int b = 0; b < 2; ++b) {
-    if (!encode<T>(&m.main[b], a.buf[b], a, NX, ny, Q) || !encode<T>(&m.lines[b], a.buf[b], a, NX, 2, Q) ||
-        !encode<T>(&m.carry[b], a.buf[b], a, CC, ny + 2, Q) || !encode<T>(&m.in2[b], a.buf[b], a, NX, ny, 2) ||
-        !encode<T>(&m.in1[b], a.buf[b], a, NX, ny, 1))
+    if (!encode<T>(&m.main[b], a.buf[b], a, NXP, ny, Q) || !encode<T>(&m.lines[b], a.buf[b], a, NXP, 2, Q) ||
+        !encode<T>(&m.carry[b], a.buf[b], a, CC, ny + 2, Q) || !encode<T>(&m.in2[b], a.buf[b], a, NXP, ny, 2) ||
+        !encode<T>(&m.in1[b], a.buf[b], a, NXP, ny, 1))
       return cudaErrorInvalidValue;
   }
   const int64_t items = (a.S0_hi - a.S0_lo + 1) * a.n1 * a.n2;
   const int gsz = (int)(items < grid ? items : grid);
-  fast3d_kernel<T, KIND><<<gsz, NT<T>, smem, s>>>(a, m);
+  kern<<<gsz, NT, smem, s>>>(a, m);
   return cudaGetLastError();
 }
 
 }  // namespace fast3d
 
-size_t fast3d_smem_bytes(int dtype, int Q) {
-  return dtype == 1 ? fast3d::smem_bytes<double>(Q) : fast3d::smem_bytes<float>(Q);
-}
-int fast3d_tile_lines(int dtype) { return dtype == 1 ? fast3d::NY<double> : fast3d::NY<float>; }
+// the instantiation this object carries (fast3d_variants.h, -DHEXS_F3_VARIANT=<id>)
+template <int ID> struct Sel3;
+#define HEXS_F3_SEL(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_)                         \
+  template <> struct Sel3<id> {                                                          \
+    using T = T_;                                                                        \
+    static constexpr int KIND = KIND_, H = H_, W0 = W0_, NY = NY_, MINB = MINB_, ZS = ZS_; \
+  };
+HEXS_FAST3D_VARIANTS(HEXS_F3_SEL)
+#undef HEXS_F3_SEL
+#define HEXS_F3_CAT2(a, b) a##b
+#define HEXS_F3_CAT(a, b) HEXS_F3_CAT2(a, b)
+using S3 = Sel3<HEXS_F3_VARIANT>;
 
-// variant id = kind * 2 + dtype for the 3D classes
-cudaError_t launch_fast3d(int variant, const Fast3DArgs& a, int /*grid: persistent*/, cudaStream_t s) {
-  switch (variant) {
-    case K_STAR3D7 * 2: return fast3d::launch_t<float, K_STAR3D7>(a, s);
-    case K_STAR3D7 * 2 + 1: return fast3d::launch_t<double, K_STAR3D7>(a, s);
-    case K_GRADIENT3D * 2: return fast3d::launch_t<float, K_GRADIENT3D>(a, s);
-    case K_GRADIENT3D * 2 + 1: return fast3d::launch_t<double, K_GRADIENT3D>(a, s);
-    case K_BOX3D27 * 2: return fast3d::launch_t<float, K_BOX3D27>(a, s);
-    case K_BOX3D27 * 2 + 1: return fast3d::launch_t<double, K_BOX3D27>(a, s);
-    default: return cudaErrorInvalidValue;
+cudaError_t HEXS_F3_CAT(launch_fast3d_v, HEXS_F3_VARIANT)(const Fast3DArgs& a, cudaStream_t s) {
+  return fast3d::launch_t<S3::T, S3::KIND, S3::H, S3::W0, S3::NY, S3::MINB, S3::ZS>(a, s);
+}
+#ifdef HEXS_F3_TIMING
+extern "C" int HEXS_F3_CAT(hexs_f3_timing_v, HEXS_F3_VARIANT)(unsigned long long* host, int reset) {
+  if (cudaMemcpyFromSymbol(host, fast3d::g_f3_tm, sizeof(fast3d::g_f3_tm)) != cudaSuccess) return -1;
+  if (reset) {
+    static unsigned long long zero[1024 * 2 * 8];
+    cudaMemcpyToSymbol(fast3d::g_f3_tm, zero, sizeof(zero));
   }
+  return 0;
+}
+#endif
+size_t HEXS_F3_CAT(fast3d_smem_v, HEXS_F3_VARIANT)() {
+  return fast3d::Lay<S3::T, fast3d::Hex<S3::H, S3::W0>::Q, S3::NY>::SMEM;
 }
 
 }  // namespace hexs

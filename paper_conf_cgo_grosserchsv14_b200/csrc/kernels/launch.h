@@ -90,7 +90,5 @@ struct Fast3DArgs {
 };
 cudaError_t launch_fast3d(int variant, const Fast3DArgs& a, int grid, cudaStream_t s);
 constexpr int kFast3DNX = 32;            // classical tile width along x of the 3D fast kernel
-int fast3d_tile_lines(int dtype);        // classical tile height along y (32 fp32, 16 fp64)
-size_t fast3d_smem_bytes(int dtype, int Q);
 
 }  // namespace hexs

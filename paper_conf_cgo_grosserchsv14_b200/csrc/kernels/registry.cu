@@ -2,6 +2,7 @@
 #include "../internal.h"
 #include "../stencil_ops.cuh"
 #include "fast2d_variants.h"
+#include "fast3d_variants.h"
 #include "launch.h"
 
 namespace hexs {
@@ -45,18 +46,36 @@ int fdtd_variant(int dtype, int h, int w0) {
   if (2 * h + 2 > 64 || W > 40 || fdtd_smem_bytes(dtype, W) > 200 * 1024) return -1;
   return dtype == 1 ? 1 : 0;
 }
-// 3D fast kernel: any (h, w0) whose two level buffers fit in shared memory
-// (2 x (w0 + 2h + 3) rows x (main + carry lines + carry columns) of one classical tile).
-int fast3d_variant(int kind, int dtype, int h, int w0) {
-  if (kind != K_STAR3D7 && kind != K_GRADIENT3D && kind != K_BOX3D27) return -1;
-  const int Q = w0 + 2 * h + 3;
-  if (fast3d_smem_bytes(dtype, Q) > 200 * 1024 || 2 * h + 2 > kMaxH) return -1;
-  return kind * 2 + dtype;
+// 3D fast kernel: the compiled (class, dtype, h, w0) instantiations of fast3d_variants.h.
+#define HEXS_F3_DECL(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_) \
+  cudaError_t launch_fast3d_v##id(const Fast3DArgs& a, cudaStream_t s);
+HEXS_FAST3D_VARIANTS(HEXS_F3_DECL)
+#undef HEXS_F3_DECL
+
+int fast3d_variant(int kind, int dtype, int h, int w0, int wy) {
+#define HEXS_F3_MATCH(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_) \
+  if (kind == KIND_ && dtype == dc && h == H_ && w0 == W0_ && (wy <= 0 || wy == NY_)) return id;
+  HEXS_FAST3D_VARIANTS(HEXS_F3_MATCH)
+#undef HEXS_F3_MATCH
+  return -1;
 }
 int fast3d_tile(int variant, int* wy, int* wx) {
-  *wy = fast3d_tile_lines(variant & 1);
+  *wy = 0;
+#define HEXS_F3_NY(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_) \
+  if (variant == id) *wy = NY_;
+  HEXS_FAST3D_VARIANTS(HEXS_F3_NY)
+#undef HEXS_F3_NY
   *wx = kFast3DNX;
-  return 0;
+  return *wy > 0 ? 0 : -1;
+}
+cudaError_t launch_fast3d(int variant, const Fast3DArgs& a, int /*grid: persistent*/, cudaStream_t s) {
+  switch (variant) {
+#define HEXS_F3_L(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_) \
+  case id: return launch_fast3d_v##id(a, s);
+    HEXS_FAST3D_VARIANTS(HEXS_F3_L)
+#undef HEXS_F3_L
+    default: return cudaErrorInvalidValue;
+  }
 }
 
 }  // namespace hexs

@@ -236,9 +236,12 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
           p->d1.n == 1 && p->d1.d == 1)
         ex = EXEC_FAST2D;
     } else {
-      p->variant = fast3d_variant(d.kind, dtype, h, w0);
+      p->variant = fast3d_variant(d.kind, dtype, h, w0, t.w[0]);
       // TMA tensor maps need 16-B aligned plane/line strides (N2 * elem % 16 == 0)
-      if (p->variant >= 0 && p->hd == 0 && (d.ext[2] * (int64_t)d.elem()) % 16 == 0) ex = EXEC_FAST3D;
+      // the kernel's hexagon is the unit-slope closed form (compile-time rows per level)
+      if (p->variant >= 0 && p->hd == 0 && (d.ext[2] * (int64_t)d.elem()) % 16 == 0 && p->d0.n == 1 &&
+          p->d0.d == 1 && p->d1.n == 1 && p->d1.d == 1)
+        ex = EXEC_FAST3D;
     }
   } else if (flags != STENCIL_EXEC_GENERIC) {
     return fail(STENCIL_E_INVALID, "stencil_plan: unknown tile.flags");
@@ -322,14 +325,18 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
   // flags and a work counter follow the ping-pong buffer in the workspace.
   p->wavefront = ((ex == EXEC_GENERIC || ex == EXEC_FAST3D) && d.dims == 3 && p->ncls == 2);
   if (p->wavefront && !p->launches.empty()) {
-    int64_t max_items = 0;
-    for (const Launch& l : p->launches)
-      max_items = std::max<int64_t>(max_items, (l.S0_hi - l.S0_lo + 1) * (l.Shi[0] - l.Slo[0] + 1) *
-                                                   (l.Shi[1] - l.Slo[1] + 1));
+    // every launch owns its flags and work counter, so one memset per stencil_run resets
+    // them all (no reset between the launches of a run)
+    int64_t n_items = 0, idx = 0;
+    for (Launch& l : p->launches) {
+      l.flag_first = n_items;
+      l.counter_idx = idx++;
+      n_items += (l.S0_hi - l.S0_lo + 1) * (l.Shi[0] - l.Slo[0] + 1) * (l.Shi[1] - l.Slo[1] + 1);
+    }
     p->flag_off = p->ws_bytes;
-    p->flag_bytes = ((size_t)max_items * sizeof(int) + 255) / 256 * 256;
-    p->counter_off = p->flag_off + p->flag_bytes;
-    p->ws_bytes = p->counter_off + 256;
+    p->counter_off = p->flag_off + ((size_t)n_items * sizeof(int) + 255) / 256 * 256;
+    p->flag_bytes = p->counter_off - p->flag_off + ((size_t)idx * 8 + 255) / 256 * 256;  // flags + counters
+    p->ws_bytes = p->flag_off + p->flag_bytes;
   }
   *out = guard.release();
   return STENCIL_OK;

@@ -115,6 +115,9 @@ stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* 
       ev_end(s);
     }
   } else {
+    if (p.wavefront)
+      HEXS_CUDA(cudaMemsetAsync(static_cast<char*>(p.ws) + p.flag_off, 0, p.flag_bytes, s),
+                "stencil_run: reset tile flags");
     for (const Launch& l : p.launches) {
       const int a_final = (l.tau0 + l.a_hi + 1 == p.tau_levels) ? l.a_hi : -1;
       const int64_t grid64 = l.S0_hi - l.S0_lo + 1;
@@ -185,9 +188,8 @@ stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* 
           a.hi[q] = p.hi[q];
         }
         char* ws = static_cast<char*>(p.ws);
-        a.flags = reinterpret_cast<int*>(ws + p.flag_off);
-        a.counter = reinterpret_cast<unsigned long long*>(ws + p.counter_off);
-        HEXS_CUDA(cudaMemsetAsync(ws + p.flag_off, 0, p.flag_bytes + 256, s), "stencil_run: reset tile flags");
+        a.flags = reinterpret_cast<int*>(ws + p.flag_off) + l.flag_first;
+        a.counter = reinterpret_cast<unsigned long long*>(ws + p.counter_off) + l.counter_idx;
         HEXS_CUDA(launch_fast3d(p.variant, a, grid, s), "stencil_run: fast3d kernel launch");
       } else {
         GenericArgs g{};
@@ -202,9 +204,8 @@ stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* 
         if (p.wavefront) {
           char* ws = static_cast<char*>(p.ws);
           g.wf = 1;
-          g.flags = reinterpret_cast<int*>(ws + p.flag_off);
-          g.counter = reinterpret_cast<unsigned long long*>(ws + p.counter_off);
-          HEXS_CUDA(cudaMemsetAsync(ws + p.flag_off, 0, p.flag_bytes + 256, s), "stencil_run: reset tile flags");
+          g.flags = reinterpret_cast<int*>(ws + p.flag_off) + l.flag_first;
+          g.counter = reinterpret_cast<unsigned long long*>(ws + p.counter_off) + l.counter_idx;
         }
         HEXS_CUDA(launch_generic(d.kind, d.dtype, g, grid, s), "stencil_run: generic kernel launch");
       }

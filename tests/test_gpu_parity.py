@@ -171,3 +171,28 @@ def test_full_size_sampled(kind):
     pts = np.array([[1, 1], [1, N - 2], [N - 2, 1], [N // 2, N // 2], [4097, 17], [1000, 8190]])
     exp = oracle.points(kind, g, T, pts)
     assert np.array_equal(got[tuple(pts.T)], exp)
+
+
+@pytest.mark.slow
+@pytest.mark.parametrize("kind", ["star3d7", "gradient3d"])
+def test_full_size_3d(kind):
+    """configs[3] (512^3, T=128) in the bench's launch configuration (auto tile, fast 3D
+    kernel): the whole grid against the oracle (OpenMP over the outer dimension; bit-exact,
+    points within a step are independent)."""
+    N, T = 512, 128
+    g = stencil_inputs.uniform((N, N, N), seed=0)
+    got, plan = _gpu_run(kind, g, T, np.float32)
+    assert plan.info["fast_kernel"] == 1
+    exp = oracle.run(kind, g, T, nthreads=oracle.max_threads())
+    assert_bitexact(got, exp, f"{kind} 512^3 T=128")
+
+
+@pytest.mark.slow
+def test_full_size_fdtd():
+    """configs[2] (fdtd-2D 8192^2, T=500) in the bench's launch configuration, whole fields."""
+    f = stencil_inputs.fields((8192, 8192), seed=0, n=3)
+    got, plan = _gpu_fdtd(f, 500, np.float32)
+    assert plan.info["fast_kernel"] == 1
+    exp = oracle.fdtd(*[x.copy() for x in f], 500, nthreads=oracle.max_threads())
+    for a, b, name in zip(got, exp, ("ex", "ey", "hz")):
+        assert_bitexact(a, b, f"fdtd 8192^2 T=500 {name}")
