@@ -44,6 +44,9 @@
 #include "launch.h"
 #include "tma.cuh"
 
+#ifndef HEXS_F3_UNROLL
+#define HEXS_F3_UNROLL 1  // 0: rolled star sweeps (smaller code; measured equal or slower)
+#endif
 #ifndef HEXS_F3_VARIANT
 #error "hex3d.cu is compiled once per fast3d variant: -DHEXS_F3_VARIANT=<id>"
 #endif
@@ -169,6 +172,19 @@ __device__ __forceinline__ void load_win(Win<T>& w, const T* const (&p)[3], int 
       w.v[l][0] = w.v[l][5] = T(0);  // never used by this stencil
     }
   }
+}
+// star / gradient: the shuffles of a row are issued one row before their selects, so the
+// shuffle latency hides behind a row of arithmetic (only the centre row's centre line needs
+// x edges: the z neighbours are centre columns)
+template <typename T> struct Edge { T l, r; };
+template <typename T>
+__device__ __forceinline__ Edge<T> edges_shfl(const Win<T>& w) {
+  return {__shfl_up_sync(0xffffffffu, w.v[1][4], 1, NQ), __shfl_down_sync(0xffffffffu, w.v[1][1], 1, NQ)};
+}
+template <typename T>
+__device__ __forceinline__ void edges_sel(Win<T>& w, const Edge<T>& e, int q) {
+  w.v[1][0] = q != 0 ? e.l : w.v[1][0];
+  w.v[1][5] = q != NQ - 1 ? e.r : w.v[1][5];
 }
 template <typename T, bool ALL_EDGES>
 __device__ __forceinline__ void edges_win(Win<T>& w, int q) {
@@ -505,25 +521,28 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
             }
             gp += plane;
           };
-          if constexpr (KIND == K_STAR3D7) {
+          if constexpr (KIND == K_STAR3D7 && HEXS_F3_UNROLL) {
             // short per-point expression: the whole sweep unrolled and software-pipelined
             // (loads of row i+3, edges of row i+2, arithmetic of row i+1)
+            // row i+1 needs its edges before step(i); rows' shuffles run one row earlier
             Win<T> w[N + 2];
             load_win<T, E27>(w[0], Pr, q);
             adv();
             load_win<T, E27>(w[1], Pr, q);
             adv();
-            edges_win<T, E27>(w[0], q);
             load_win<T, E27>(w[2], Pr, q);
             adv();
-            edges_win<T, E27>(w[1], q);
+            Edge<T> e1 = edges_shfl(w[1]);
+            Edge<T> e2 = edges_shfl(w[2]);
 #pragma unroll
             for (int i = 0; i < N; ++i) {
               if (i + 3 < N + 2) {
                 load_win<T, E27>(w[i + 3], Pr, q);
                 adv();
               }
-              edges_win<T, E27>(w[i + 2], q);
+              edges_sel(w[i + 1], e1, q);
+              e1 = e2;
+              if (i + 3 < N + 2) e2 = edges_shfl(w[i + 3]);
               step(i, w[i], w[i + 1], w[i + 2]);
             }
           } else {

@@ -147,8 +147,11 @@ class SlabRunner:
         return (s.local_extent - (s.own_hi - s.own_lo)) / max(1, s.own_hi - s.own_lo)
 
 
-def bench_main(args, cfg, configs, metric):
-    """bench.py --gpus N under torchrun: weak scaling, each rank owns the config's grid."""
+def bench_main(args, cfg, configs, metric, helpers=None):
+    """bench.py --gpus N under torchrun: weak scaling, each rank owns the config's grid.
+    `helpers` is the bench module (clock sampler, roofline model, peaks)."""
+    import stencil_inputs
+
     kind, ext, T, cname = configs[cfg]
     rank = int(os.environ["RANK"])
     world = int(os.environ["WORLD_SIZE"])
@@ -156,9 +159,8 @@ def bench_main(args, cfg, configs, metric):
     torch.cuda.set_device(local_rank)
     dist.init_process_group("nccl", device_id=torch.device("cuda", local_rank))
     gext = (ext[0] * world,) + tuple(ext[1:])
-    D = int(os.environ.get("HEXS_TIME_BLOCK", "64"))
+    D = int(os.environ.get("HEXS_TIME_BLOCK", "128"))
     runner = SlabRunner(kind, gext, T, D=D)
-    import stencil_inputs
 
     # each rank generates only its local planes of the global synthetic grid (same recipe)
     s = runner.slab
@@ -166,7 +168,8 @@ def bench_main(args, cfg, configs, metric):
     for e in gext[1:]:
         plane *= e
     local_np = stencil_inputs.uniform((s.local_extent,) + tuple(gext[1:]), seed=0, offset=s.loc_lo * plane)
-    local0 = torch.from_numpy(local_np).cuda()
+    host_in = torch.from_numpy(local_np).pin_memory()
+    local0 = host_in.cuda()
     local = torch.empty_like(local0)
     stream = torch.cuda.current_stream()
 
@@ -179,16 +182,60 @@ def bench_main(args, cfg, configs, metric):
     torch.cuda.synchronize()
     dist.barrier()
     e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    sampler = helpers.ClockSampler(local_rank) if helpers is not None else None
+    if sampler is not None:
+        sampler.__enter__()
     e0.record(stream)
     for _ in range(args.steps):
         step()
     e1.record(stream)
     torch.cuda.synchronize()
+    if sampler is not None:
+        sampler.__exit__(None, None, None)
     ms = torch.tensor([e0.elapsed_time(e1) / args.steps], device="cuda")
     dist.all_reduce(ms, op=dist.ReduceOp.MAX)
     ms = float(ms.item())
     value = runner.updates() / (ms * 1e-3) / 1e9
+
+    # end to end through the public API: pinned H2D of the rank's slab, the run (halo
+    # exchanges included), D2H of the owned planes
+    lo, hi = s.own_local
+    host_out = torch.empty_like(host_in[lo:hi]).pin_memory()
+    dist.barrier()
+    torch.cuda.synchronize()
+    f0, f1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    f0.record(stream)
+    for _ in range(args.steps):
+        local.copy_(host_in, non_blocking=True)
+        runner.run(local)
+        host_out.copy_(local[lo:hi], non_blocking=True)
+    f1.record(stream)
+    torch.cuda.synchronize()
+    e2e_ms = torch.tensor([f0.elapsed_time(f1) / args.steps], device="cuda")
+    dist.all_reduce(e2e_ms, op=dist.ReduceOp.MAX)
+    e2e_ms = float(e2e_ms.item())
+
+    # phase-kernel roofline of the main block plan (algorithmic bytes / measured launch time)
+    roof = None
+    plan = runner._plans.get(runner.D)
+    launches = sum(runner._plans[b].info["n_launches"] for b in runner.blocks)
+    if plan is not None and helpers is not None:
+        plan.profile(1)
+        step()
+        prof = plan.profile_read()
+        plan.profile(0)
+        info = plan.info
+        bpu = helpers.bytes_per_update_tiled(info, 4, plan)
+        avg = prof["kernel_ms"] / max(1, prof["launches"])
+        alg = info["updates"] / info["n_launches"] * bpu
+        peak, peak_src = helpers.load_peaks()
+        roof = {"bound": "hbm", "achieved": alg / (avg * 1e-3) / 1e9, "peak": peak, "unit": "GB/s",
+                "frac": alg / (avg * 1e-3) / 1e9 / peak, "traffic": None, "peak_source": peak_src,
+                "kernel": helpers.KERNEL_NAMES.get(plan.executor_name, plan.executor_name),
+                "bytes_per_update": bpu, "avg_launch_ms": avg}
     if rank == 0:
+        nbytes_in = host_in.numel() * host_in.element_size()
+        nbytes_out = host_out.numel() * host_out.element_size()
         line = {"metric": metric, "value": value, "unit": "GStencil-updates/s", "n_gpus": world,
                 "steps": args.steps, "warmup": args.warmup, "ms_per_step": ms,
                 "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "f32",
@@ -196,7 +243,14 @@ def bench_main(args, cfg, configs, metric):
                 "config": {"workload": cname + f" weak-scaled to {gext[0]} planes over {world} GPUs",
                            "kind": kind, "extents": list(gext), "T": T, "time_block": runner.D,
                            "ghost_planes": runner.slab.ghost,
-                           "redundant_fraction": runner.redundant_fraction()},
-                "gpu_launches": None}
+                           "redundant_fraction": runner.redundant_fraction(),
+                           "l2": "inputs larger than L2 (per-rank slab > 126 MB)"},
+                "roofline": roof,
+                "cpu_baseline": None,
+                "e2e": {"value": runner.updates() / (e2e_ms * 1e-3) / 1e9, "unit": "GStencil-updates/s",
+                        "h2d_bytes_per_step": nbytes_in * world, "d2h_bytes_per_step": nbytes_out * world,
+                        "ms_per_step": e2e_ms},
+                "gpu_launches": launches * args.steps,
+                "clocks": sampler.summary() if sampler is not None else None}
         print(json.dumps(line), flush=True)
     dist.destroy_process_group()
