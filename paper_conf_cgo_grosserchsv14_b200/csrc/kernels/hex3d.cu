@@ -58,7 +58,16 @@ constexpr int NX = kFast3DNX;  // tile columns (x)
 constexpr int NXP = NX + 4;    // shared-memory line pitch (spreads the per-line edge loads over banks)
 constexpr int NQ = NX / 4;     // column quads: one 8-lane group
 constexpr int SIGMA = 4;       // x skew per level
-constexpr int CC = 8;          // carry-area columns (x = X0 - 4a - 4 .. X0 - 4a + 3)
+// Carry areas (the predecessor tiles' values): the carry-column quad (main-frame m = -4 .. -1)
+// and the edge column (m = -5, element 3 of its quad) in areas of 16-B lines, and 2 carry lines.
+// Each TMA box starts a few lines early (SC, SL) and rows are padded to 8-chunk multiples, so
+// that lane 0's carry quad lands in the one 16-B bank slot its 8-lane group leaves free in the
+// same LDS.128 (conflict-free; a TMA destination itself must stay 128-B aligned).
+// (fp32 bank geometry; the fp64 variants keep the dense 2-line / NY+2-line areas)
+template <typename T> constexpr int SC = sizeof(T) == 4 ? 5 : 0;  // line shift of the carry boxes
+template <typename T> constexpr int SL = sizeof(T) == 4 ? 6 : 0;  // line shift of the carry-line box
+template <typename T> constexpr int LR = sizeof(T) == 4 ? 8 : 2;  // lines per row, carry-line area
+template <typename T> constexpr int CLP = sizeof(T) == 4 ? 8 : 2; // extra lines per row, carry areas
 
 // Hexagon of a radius-1 single-statement stencil (delta0 = delta1 = 1): rows b of level a
 // (SURVEY §8(a) closed form of eqs. (6)-(13)); buffer rows b = -1 .. 2h + w0 + 1.
@@ -73,26 +82,31 @@ template <int H, int W0> struct Hex {
 };
 
 constexpr int al128(int bytes) { return (bytes + 127) / 128 * 128; }
-// One buffer (level a's input = level a-1 values), Q rows (buffer row rr = b + 1):
-//   main  [Q][NY][NXP]    own region: y = Y0 - a + 1 + l, x = X0 - 4a + 4 + m
-//   lines [Q][2][NXP]     carry lines: y = Y0 - a - 1 + l, x as main
-//   carry [Q][NY+2][CC]   carry columns: y = Y0 - a - 1 + l, x = X0 - 4a - 4 + c
+// One buffer (level a's input = level a-1 values), Q rows (buffer row rr = b + 1), input-frame
+// line L' = 0 .. NY+1 (y = Y0 - a - 1 + L'):
+//   main  [Q][NY][NXP]   own region: lines L' = 2 + l, x = X0 - 4a + 4 + m
+//   lines [Q][LR][NXP]   carry lines: L' = l - SL (l = SL, SL+1), x as main
+//   carry [Q][CL][4]     carry quad: L' = l - SC, x = X0 - 4a + c      (m = c - 4)
+//   edge  [Q][CL][4]     edge column: L' = l - SC, x = X0 - 4a - 4 + c (c = 3: m = -5)
 // Each area starts 128-B aligned (TMA destinations).  Offsets in elements.
 template <typename T, int Q, int NY> struct Lay {
-  static constexpr int MAIN = NY * NXP, LINES = 2 * NXP, CARRY = (NY + 2) * CC;
+  static constexpr int CL = NY + CLP<T>;  // lines per row of the carry / edge areas (>= NY + 2 + SC)
+  static constexpr int MAIN = NY * NXP, LINES = LR<T> * NXP, CARRY = CL * 4;
   static constexpr int LINES_OFF = al128(Q * MAIN * (int)sizeof(T)) / (int)sizeof(T);
   static constexpr int CARRY_OFF = al128((LINES_OFF + Q * LINES) * (int)sizeof(T)) / (int)sizeof(T);
-  static constexpr int BUF = al128((CARRY_OFF + Q * CARRY) * (int)sizeof(T)) / (int)sizeof(T);
+  static constexpr int EDGE_OFF = al128((CARRY_OFF + Q * CARRY) * (int)sizeof(T)) / (int)sizeof(T);
+  static constexpr int BUF = al128((EDGE_OFF + Q * CARRY) * (int)sizeof(T)) / (int)sizeof(T);
   static constexpr size_t SMEM = 2 * (size_t)BUF * sizeof(T);
-  static constexpr uint32_t FIRST_BYTES = (uint32_t)(Q * (MAIN + LINES + CARRY) * sizeof(T));
-  static constexpr uint32_t CARRY_BYTES = (uint32_t)(Q * (LINES + CARRY) * sizeof(T));
+  static_assert(SMEM + 1024 <= 227 * 1024, "two level buffers must fit the 227 KB opt-in shared memory");
+  static constexpr uint32_t FIRST_BYTES = (uint32_t)(Q * (MAIN + LINES + 2 * CARRY) * sizeof(T));
+  static constexpr uint32_t CARRY_BYTES = (uint32_t)(Q * (LINES + 2 * CARRY) * sizeof(T));
   static constexpr uint32_t ROW_BYTES = (uint32_t)(MAIN * sizeof(T));
 };
 
 struct Maps {
   CUtensorMap main[2];   // box {NXP, NY, Q}
-  CUtensorMap lines[2];  // box {NXP, 2, Q}
-  CUtensorMap carry[2];  // box {CC, NY+2, Q}
+  CUtensorMap lines[2];  // box {NXP, LR, Q}
+  CUtensorMap carry[2];  // box {4, NY+8, Q} (carry quads and edge columns)
   CUtensorMap in2[2];    // box {NXP, NY, 2}
   CUtensorMap in1[2];    // box {NXP, NY, 1}
 };
@@ -154,7 +168,7 @@ template <typename T> struct Win { T v[3][6]; };
 // load_win issues the loads (vector quads; the group's outer lanes also load their edge
 // column with a predicated scalar load), edges_win completes the edges by shuffle.
 template <typename T, bool ALL_EDGES>  // star / gradient stencils need the centre line's edges only
-__device__ __forceinline__ void load_win(Win<T>& w, const T* const (&p)[3], int q) {
+__device__ __forceinline__ void load_win(Win<T>& w, const T* const (&p)[3], int q, int eo) {
 #pragma unroll
   for (int l = 0; l < 3; ++l) {
     if constexpr (sizeof(T) == 4) {
@@ -166,7 +180,7 @@ __device__ __forceinline__ void load_win(Win<T>& w, const T* const (&p)[3], int 
       w.v[l][1] = u0.x; w.v[l][2] = u0.y; w.v[l][3] = u1.x; w.v[l][4] = u1.y;
     }
     if (ALL_EDGES || l == 1) {
-      w.v[l][0] = lds_if(q == 0, p[l] - 1, T(0));
+      w.v[l][0] = lds_if(q == 0, p[l] + eo, T(0));  // lane 0: the edge area
       w.v[l][5] = lds_if(q == NQ - 1, p[l] + 4, T(0));
     } else {
       w.v[l][0] = w.v[l][5] = T(0);  // never used by this stencil
@@ -256,16 +270,17 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
   for (int k = 0; k < 3; ++k) {
     const int l = ly + k;
     if (q == 0) {
-      woff[k] = LY::CARRY_OFF + l * CC + 4;
+      woff[k] = LY::CARRY_OFF + (l + SC<T>) * 4;
       wpitch[k] = LY::CARRY;
     } else if (l < 2) {
-      woff[k] = LY::LINES_OFF + l * NXP + 4 * q - 4;
+      woff[k] = LY::LINES_OFF + (l + SL<T>) * NXP + 4 * q - 4;
       wpitch[k] = LY::LINES;
     } else {
       woff[k] = (l - 2) * NXP + 4 * q - 4;
       wpitch[k] = LY::MAIN;
     }
   }
+  const int eo = q == 0 ? LY::EDGE_OFF - LY::CARRY_OFF + 3 : -1;  // left edge relative to the quad
   const int sts_off = ly * NXP + 4 * q;                  // + row * MAIN in the output buffer
   const bool cthr = (ly >= LNY - 2) || (q >= NQ - 2);   // writes its successors' carries
 
@@ -313,8 +328,9 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
     T* B = buf_of(b);
     mbar_arrive_expect_tx(&full[b], LY::FIRST_BYTES);
     tma_3d(B, &mp.main[par], xo + 4, yo + 1, z0, &full[b]);
-    tma_3d(B + LY::LINES_OFF, &mp.lines[par], xo + 4, yo - 1, z0, &full[b]);
-    tma_3d(B + LY::CARRY_OFF, &mp.carry[par], xo - 4, yo - 1, z0, &full[b]);
+    tma_3d(B + LY::LINES_OFF, &mp.lines[par], xo + 4, yo - 1 - SL<T>, z0, &full[b]);
+    tma_3d(B + LY::CARRY_OFF, &mp.carry[par], xo, yo - 1 - SC<T>, z0, &full[b]);
+    tma_3d(B + LY::EDGE_OFF, &mp.carry[par], xo - 4, yo - 1 - SC<T>, z0, &full[b]);
   };
   // In rows of level a: buffer rows level a reads ([lo(a)-1, hi(a)+1]) that level a-1 does
   // not compute (0, 1 or 2 per side)
@@ -355,8 +371,9 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
     tile_origin(it, i0, X0, Y0);
     const int b = a & 1, par = (int)((g.tau0 + a) & 1);
     const int z0 = (int)(i0 - 1), xo = X0 - SIGMA * a, yo = Y0 - a;
-    tma_3d(buf_of(b) + LY::LINES_OFF, &mp.lines[par], xo + 4, yo - 1, z0, &full[b]);
-    tma_3d(buf_of(b) + LY::CARRY_OFF, &mp.carry[par], xo - 4, yo - 1, z0, &full[b]);
+    tma_3d(buf_of(b) + LY::LINES_OFF, &mp.lines[par], xo + 4, yo - 1 - SL<T>, z0, &full[b]);
+    tma_3d(buf_of(b) + LY::CARRY_OFF, &mp.carry[par], xo, yo - 1 - SC<T>, z0, &full[b]);
+    tma_3d(buf_of(b) + LY::EDGE_OFF, &mp.carry[par], xo - 4, yo - 1 - SC<T>, z0, &full[b]);
   };
 
   F3_TM_DECL
@@ -526,18 +543,18 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
             // (loads of row i+3, edges of row i+2, arithmetic of row i+1)
             // row i+1 needs its edges before step(i); rows' shuffles run one row earlier
             Win<T> w[N + 2];
-            load_win<T, E27>(w[0], Pr, q);
+            load_win<T, E27>(w[0], Pr, q, eo);
             adv();
-            load_win<T, E27>(w[1], Pr, q);
+            load_win<T, E27>(w[1], Pr, q, eo);
             adv();
-            load_win<T, E27>(w[2], Pr, q);
+            load_win<T, E27>(w[2], Pr, q, eo);
             adv();
             Edge<T> e1 = edges_shfl(w[1]);
             Edge<T> e2 = edges_shfl(w[2]);
 #pragma unroll
             for (int i = 0; i < N; ++i) {
               if (i + 3 < N + 2) {
-                load_win<T, E27>(w[i + 3], Pr, q);
+                load_win<T, E27>(w[i + 3], Pr, q, eo);
                 adv();
               }
               edges_sel(w[i + 1], e1, q);
@@ -550,7 +567,7 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
             // 3-row register window keeps the level's code small enough for the i-cache
             Win<T> wa, wb, wc;
             auto ld = [&](Win<T>& w) {
-              load_win<T, E27>(w, Pr, q);
+              load_win<T, E27>(w, Pr, q, eo);
               adv();
               edges_win<T, E27>(w, q);
             };
@@ -640,8 +657,8 @@ cudaError_t launch_t(const Fast3DArgs& a, cudaStream_t s) {
   Maps m;
   const uint32_t Q = (uint32_t)a.Q, ny = (uint32_t)NY;
   for (int b = 0; b < 2; ++b) {
-    if (!encode<T>(&m.main[b], a.buf[b], a, NXP, ny, Q) || !encode<T>(&m.lines[b], a.buf[b], a, NXP, 2, Q) ||
-        !encode<T>(&m.carry[b], a.buf[b], a, CC, ny + 2, Q) || !encode<T>(&m.in2[b], a.buf[b], a, NXP, ny, 2) ||
+    if (!encode<T>(&m.main[b], a.buf[b], a, NXP, ny, Q) || !encode<T>(&m.lines[b], a.buf[b], a, NXP, LR<T>, Q) ||
+        !encode<T>(&m.carry[b], a.buf[b], a, 4, ny + CLP<T>, Q) || !encode<T>(&m.in2[b], a.buf[b], a, NXP, ny, 2) ||
         !encode<T>(&m.in1[b], a.buf[b], a, NXP, ny, 1))
       return cudaErrorInvalidValue;
   }
