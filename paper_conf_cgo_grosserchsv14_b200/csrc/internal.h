@@ -109,7 +109,7 @@ bool schedule_of(const Plan& p, int64_t tau, const int64_t* s, int64_t* sched);
 stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* stream);
 
 // Fast-kernel registry (kernels/*.cu): returns variant id >= 0 or -1 if not instantiated.
-int fast2d_variant(int kind, int dtype, int h, int w0);
+int fast2d_variant(int kind, int dtype, int h, int w0, int w1);
 int fast2d_chunk_width(int variant);  // classical tile width w1 the kernel streams
 int fdtd_variant(int dtype, int h, int w0);
 int fast3d_variant(int kind, int dtype, int h, int w0, int wy);

@@ -18,5 +18,9 @@
   X(11, 0, float, K_STAR2D5, 3, 5, 4)            \
   X(12, 0, float, K_STAR2D5, 4, 5, 4)            \
   X(13, 0, float, K_JACOBI2D5, 1, 3, 4)          \
-  X(14, 0, float, K_BOX2D9, 3, 5, 4)
-#define HEXS_FAST2D_COUNT 15
+  X(14, 0, float, K_BOX2D9, 3, 5, 4)             \
+  X(15, 0, float, K_BOX2D9, 2, 5, 4)             \
+  X(16, 0, float, K_BOX2D9, 2, 7, 4)             \
+  X(17, 0, float, K_BOX2D9, 4, 5, 4)             \
+  X(18, 0, float, K_BOX2D9, 3, 7, 8)
+#define HEXS_FAST2D_COUNT 19

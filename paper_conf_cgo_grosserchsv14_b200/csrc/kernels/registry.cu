@@ -13,9 +13,10 @@ namespace hexs {
 HEXS_FAST2D_VARIANTS(HEXS_DECL)
 #undef HEXS_DECL
 
-int fast2d_variant(int kind, int dtype, int h, int w0) {
-#define HEXS_MATCH(id, dc, T_, KIND_, H_, W0_, NW_) \
-  if (kind == KIND_ && dtype == dc && h == H_ && w0 == W0_) return id;
+int fast2d_variant(int kind, int dtype, int h, int w0, int w1) {
+#define HEXS_MATCH(id, dc, T_, KIND_, H_, W0_, NW_)                  \
+  if (kind == KIND_ && dtype == dc && h == H_ && w0 == W0_ &&         \
+      (w1 <= 0 || w1 == NW_ * 32 * (int)(16 / sizeof(T_)))) return id;
   HEXS_FAST2D_VARIANTS(HEXS_MATCH)
 #undef HEXS_MATCH
   return -1;

@@ -184,7 +184,11 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
       auto Wof = [&](int w) { return (int64_t)2 * w + 2 + h + h / 2; };
       while (w0 < 12 && (d.ext[0] + Wof(w0) - 1) / Wof(w0) + 1 > slots) ++w0;
     } else if (d.dims == 2) {
-      h = 3; w0 = 7;  // best measured on B200 (profiles/)
+      // best measured on B200 (profiles/round1/tile_sweep_*.txt); the 9-point
+      // box takes the shallower hexagon: its unrolled level bodies otherwise overflow the
+      // instruction cache (ncu stall "no_instruction")
+      h = 3; w0 = 7;
+      if (d.kind == STENCIL_BOX2D9 && dtype == STENCIL_F32) h = 2;
     } else {
       h = 2; w0 = 7;  // Table 4 setup
     }
@@ -231,7 +235,7 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
       // the ring is filled by 16-B cp.async: row starts must be 16-B aligned
       if (p->variant >= 0 && p->hd == 0 && (d.ext[1] * (int64_t)d.elem()) % 16 == 0) ex = EXEC_FDTD;
     } else if (d.dims == 2) {
-      p->variant = fast2d_variant(d.kind, dtype, h, w0);
+      p->variant = fast2d_variant(d.kind, dtype, h, w0, t.w[0]);
       if (p->variant >= 0 && p->hd == 0 && p->dcls[0] == 1 && p->d0.n == 1 && p->d0.d == 1 &&
           p->d1.n == 1 && p->d1.d == 1)
         ex = EXEC_FAST2D;
