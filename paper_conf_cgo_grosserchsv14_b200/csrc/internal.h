@@ -114,5 +114,6 @@ int fast2d_chunk_width(int variant);  // classical tile width w1 the kernel stre
 int fdtd_variant(int dtype, int h, int w0);
 int fast3d_variant(int kind, int dtype, int h, int w0, int wy);
 int fast3d_tile(int variant, int* wy, int* wx);
+bool fast3d_variant_matches(int variant, int kind, int dtype, int h, int w0);
 
 }  // namespace hexs

@@ -538,7 +538,7 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
             }
             gp += plane;
           };
-          if constexpr (KIND == K_STAR3D7 && HEXS_F3_UNROLL) {
+          if constexpr (KIND == K_STAR3D7 && HEXS_F3_UNROLL && ZS == 1) {
             // short per-point expression: the whole sweep unrolled and software-pipelined
             // (loads of row i+3, edges of row i+2, arithmetic of row i+1)
             // row i+1 needs its edges before step(i); rows' shuffles run one row earlier

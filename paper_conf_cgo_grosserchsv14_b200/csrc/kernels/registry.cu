@@ -60,6 +60,13 @@ int fast3d_variant(int kind, int dtype, int h, int w0, int wy) {
 #undef HEXS_F3_MATCH
   return -1;
 }
+bool fast3d_variant_matches(int variant, int kind, int dtype, int h, int w0) {
+#define HEXS_F3_IS(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_) \
+  if (variant == id) return kind == KIND_ && dtype == dc && h == H_ && w0 == W0_;
+  HEXS_FAST3D_VARIANTS(HEXS_F3_IS)
+#undef HEXS_F3_IS
+  return false;
+}
 int fast3d_tile(int variant, int* wy, int* wx) {
   *wy = 0;
 #define HEXS_F3_NY(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_) \

@@ -11,6 +11,7 @@
 //   classical tiling eqs. (14)-(17) with u = the local box row
 //   host loop "repeatedly iterating over two CUDA kernels"
 #include <algorithm>
+#include <cstdlib>
 #include <climits>
 #include <cmath>
 #include <memory>
@@ -241,6 +242,11 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
         ex = EXEC_FAST2D;
     } else {
       p->variant = fast3d_variant(d.kind, dtype, h, w0, t.w[0]);
+      // tuning aid: HEXS_F3_FORCE_VARIANT=<id> picks a compiled variant of the same shape
+      if (const char* fv = std::getenv("HEXS_F3_FORCE_VARIANT")) {
+        const int id = std::atoi(fv);
+        if (id >= 0 && fast3d_variant_matches(id, d.kind, dtype, h, w0)) p->variant = id;
+      }
       // TMA tensor maps need 16-B aligned plane/line strides (N2 * elem % 16 == 0)
       // the kernel's hexagon is the unit-slope closed form (compile-time rows per level)
       if (p->variant >= 0 && p->hd == 0 && (d.ext[2] * (int64_t)d.elem()) % 16 == 0 && p->d0.n == 1 &&
