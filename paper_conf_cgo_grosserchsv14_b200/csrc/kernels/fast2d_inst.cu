@@ -20,10 +20,10 @@ HEXS_FAST2D_VARIANTS(HEXS_SEL)
 using KSel = Sel<HEXS_VARIANT>::K;
 
 // Full-time hexagons on 16-B aligned rows: TMA-staged In rows (the hot kernel).
-__global__ void __launch_bounds__(KSel::NT * KSel::TG, KSel::MINB / KSel::TG)
+__global__ void __launch_bounds__(KSel::NT, KSel::MINB)
 HEXS_CAT(fast2d_kernel_v, HEXS_VARIANT)(const __grid_constant__ Fast2DArgs g) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
-  KSel::run_tma(g, reinterpret_cast<KSel::Smem*>(smem_raw));
+  KSel::run_tma(g, *reinterpret_cast<KSel::Smem*>(smem_raw));
 }
 // Full-time hexagons on unaligned rows (direct loads).
 __global__ void __launch_bounds__(KSel::NT, 1)
@@ -40,10 +40,10 @@ HEXS_CAT(fast2d_kernel_tcut_v, HEXS_VARIANT)(const __grid_constant__ Fast2DArgs 
 
 cudaError_t HEXS_CAT(launch_fast2d_v, HEXS_VARIANT)(const Fast2DArgs& a, int grid, cudaStream_t s) {
   static bool attr_set = false;
-  const int smem = (int)sizeof(KSel::Smem), smem_g = smem * KSel::TG;
+  const int smem = (int)sizeof(KSel::Smem);
   if (!attr_set) {
     cudaError_t e = cudaFuncSetAttribute(HEXS_CAT(fast2d_kernel_v, HEXS_VARIANT),
-                                         cudaFuncAttributeMaxDynamicSharedMemorySize, smem_g);
+                                         cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
     if (e == cudaSuccess)
       e = cudaFuncSetAttribute(HEXS_CAT(fast2d_kernel_unaligned_v, HEXS_VARIANT),
                                cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
@@ -57,7 +57,7 @@ cudaError_t HEXS_CAT(launch_fast2d_v, HEXS_VARIANT)(const Fast2DArgs& a, int gri
   if (a.a_lo > 0 || a.a_hi < KSel::L - 1)
     HEXS_CAT(fast2d_kernel_tcut_v, HEXS_VARIANT)<<<grid, KSel::NT, smem, s>>>(a);
   else if (aligned)
-    HEXS_CAT(fast2d_kernel_v, HEXS_VARIANT)<<<(grid + KSel::TG - 1) / KSel::TG, KSel::NT * KSel::TG, smem_g, s>>>(a);
+    HEXS_CAT(fast2d_kernel_v, HEXS_VARIANT)<<<grid, KSel::NT, smem, s>>>(a);
   else
     HEXS_CAT(fast2d_kernel_unaligned_v, HEXS_VARIANT)<<<grid, KSel::NT, smem, s>>>(a);
   return cudaGetLastError();

@@ -153,27 +153,36 @@ __global__ void __launch_bounds__(NT, 2) fdtd_kernel(const __grid_constant__ Fdt
       const int st = lv[l][0], blo = lv[l][1], bhi = lv[l][2];
       const int j = k * C - (g.a_lo + l) + col;
       if (j >= lv[l][3] && j <= lv[l][4]) {
+        // 32-bit shared-memory element offsets (one IADD per row step instead of 64-bit
+        // pointer arithmetic); row b of field f at (f*R + b + 1) * RC + ring column
         const int cj = (j + C) & (RC - 1);
         const int b0 = blo + rpar;
+        int o = (b0 + 1) * RC + cj;  // row b0 of a field, relative to its first row
+        constexpr int STEP = RP * RC;
         if (st == 0) {  // ey[i][j] -= ce * (hz[i][j] - hz[i-1][j])
-          T* __restrict__ pe = rey + cj + b0 * RC;
-          const T* __restrict__ ph = rhz + cj + b0 * RC;
 #pragma unroll 4
-          for (int b = b0; b <= bhi; b += RP, pe += RP * RC, ph += RP * RC) *pe = fdtd_ey<T>(*pe, ph[0], ph[-RC], cf);
+          for (int b = b0; b <= bhi; b += RP, o += STEP) {
+            T* pe = ring + R * RC + o;
+            const T* ph = ring + 2 * R * RC + o;
+            *pe = fdtd_ey<T>(*pe, ph[0], ph[-RC], cf);
+          }
         } else if (st == 1) {  // ex[i][j] -= ce * (hz[i][j] - hz[i][j-1])
           const int dm = ((j - 1 + C) & (RC - 1)) - cj;  // column j-1 relative to j in the ring
-          T* __restrict__ px = rex + cj + b0 * RC;
-          const T* __restrict__ ph = rhz + cj + b0 * RC;
 #pragma unroll 4
-          for (int b = b0; b <= bhi; b += RP, px += RP * RC, ph += RP * RC) *px = fdtd_ex<T>(*px, ph[0], ph[dm], cf);
+          for (int b = b0; b <= bhi; b += RP, o += STEP) {
+            T* px = ring + o;
+            const T* ph = ring + 2 * R * RC + o;
+            *px = fdtd_ex<T>(*px, ph[0], ph[dm], cf);
+          }
         } else {  // hz[i][j] -= ch * (((ex[i][j+1] - ex[i][j]) + ey[i+1][j]) - ey[i][j])
           const int dp = ((j + 1 + C) & (RC - 1)) - cj;  // column j+1 relative to j in the ring
-          T* __restrict__ ph = rhz + cj + b0 * RC;
-          const T* __restrict__ px = rex + cj + b0 * RC;
-          const T* __restrict__ pe = rey + cj + b0 * RC;
 #pragma unroll 4
-          for (int b = b0; b <= bhi; b += RP, ph += RP * RC, px += RP * RC, pe += RP * RC)
+          for (int b = b0; b <= bhi; b += RP, o += STEP) {
+            T* ph = ring + 2 * R * RC + o;
+            const T* px = ring + o;
+            const T* pe = ring + R * RC + o;
             *ph = fdtd_hz<T>(*ph, px[dp], px[0], pe[RC], pe[0], cf);
+          }
         }
       }
       __syncthreads();
@@ -187,9 +196,11 @@ __global__ void __launch_bounds__(NT, 2) fdtd_kernel(const __grid_constant__ Fdt
       const int cj = (j + C) & (RC - 1);
 #pragma unroll
       for (int f = 0; f < 3; ++f) {
-        const T* sp = (f == 0 ? rex : (f == 1 ? rey : rhz)) + cj;
-        T* gp = F[f] + (i0 * N1 + j);
-        for (int b = mlo[f] + rpar; b <= mhi[f]; b += RP) gp[b * N1] = sp[b * RC];
+        const int b0 = mlo[f] + rpar;
+        const T* sp = (f == 0 ? rex : (f == 1 ? rey : rhz)) + cj + b0 * RC;
+        T* gp = F[f] + ((i0 + b0) * N1 + j);
+        const int64_t gstep = RP * N1;
+        for (int b = b0; b <= mhi[f]; b += RP, sp += RP * RC, gp += gstep) *gp = *sp;
       }
     }
     __syncthreads();  // the write-back reads ring slots the next stage() overwrites

@@ -39,17 +39,12 @@
 #ifndef HEXS_MERGE_ROWP
 #define HEXS_MERGE_ROWP 1
 #endif
-#ifndef HEXS_TMA_GROUP
-#define HEXS_TMA_GROUP 0  // 1 (MINB hexagons per CTA in lockstep) measured 1514 -> 1236 GUp/s star2d5
-#endif
 #ifndef HEXS_MERGE_COLP
 #define HEXS_MERGE_COLP 0  // 1 measured slower: 1514 -> 1250 GUp/s star2d5
 #endif
 
 namespace hexs {
 namespace fast2d {
-
-__device__ __forceinline__ int64_t min64(int64_t a, int64_t b) { return a < b ? a : b; }
 
 // Compile-time loop: f(std::integral_constant<int, I>) for I in [A, N).
 template <int A, int N, class F>
@@ -87,10 +82,6 @@ struct Kernel {
   static constexpr int NT = NW * 32;
   static constexpr int C = NT * V;           // super-chunk width (classical tile w1)
   static constexpr int MINB = sizeof(T) == 8 ? 2 : 3;  // resident CTAs/SM the register budget targets
-  // Full-time TMA tiles: MINB hexagons per CTA (one 4-warp group each, in lockstep), so every
-  // warp of an SM executes the same level body at the same time: one instruction stream per SM
-  // instead of MINB CTAs thrashing the instruction cache at different points of the body.
-  static constexpr int TG = HEXS_TMA_GROUP ? MINB : 1;
   static constexpr int NIN = W0 + 4 * H + 5; // In rows per chunk (= In values per column)
   static constexpr int SW = C + 8;           // staged row width (elements), 16-B granular
 
@@ -184,7 +175,7 @@ struct Kernel {
   template <bool TMA, bool ROWP, bool COLP, bool TCUT>
   static __device__ __forceinline__ void chunk(const Fast2DArgs& g, Smem& sm, int64_t k, int64_t K,
                                                int64_t i0, const Coef<T>& cf) {
-    const int tid = threadIdx.x % NT, lane = tid & 31, warp = tid >> 5;  // within the hexagon's group
+    const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
     const int64_t N0 = g.N0, N1 = g.N1;
     T in[Q][V + 2];  // input array of the current level: [row][halo0, halo1, own V]
 #pragma unroll
@@ -325,24 +316,19 @@ struct Kernel {
   }
 
   // Full-time tiles, 16-B aligned rows: TMA-staged In rows.
-  static __device__ __forceinline__ void run_tma(const Fast2DArgs& g, Smem* sms) {
-    // group grp of the CTA runs hexagon S0 (a group past the launch's last hexagon repeats it:
-    // identical values, identical stores, so the groups stay in lockstep)
-    const int grp = threadIdx.x / NT;
-    Smem& sm = sms[grp];
-    const int64_t S0 = min64(g.S0_lo + (int64_t)blockIdx.x * TG + grp, g.S0_hi);
+  static __device__ __forceinline__ void run_tma(const Fast2DArgs& g, Smem& sm) {
+    const int64_t S0 = g.S0_lo + blockIdx.x;
     const int64_t i0 = S0 * g.W - g.row_off;  // global row of local row b = 0
     const Coef<T> cf{(T)g.k0, (T)g.k1};
     const bool rowpart = (i0 - 1 < 1) || (i0 + R > g.N0 - 2);
     const int64_t K = n_chunks(g);
-    const bool leader = threadIdx.x % NT == 0;
-    if (leader) {
+    if (threadIdx.x == 0) {
 #pragma unroll
       for (int a = 0; a < L; ++a) mbar_init(&sm.mbar[a], 1);
       mbar_fence_init();
     }
     __syncthreads();
-    if (leader) {
+    if (threadIdx.x == 0) {
 #pragma unroll
       for (int a = 0; a < L; ++a) issue_level(g, sm, 0, a, i0);
     }

@@ -51,7 +51,7 @@ struct Fast2DArgs {
   int64_t N0, N1;
   int64_t tau0;
   int a_lo, a_hi, a_final;  // a_final: level whose outputs are level T_steps (-1: none)
-  int64_t S0_lo, S0_hi, row_off;
+  int64_t S0_lo, row_off;
   int W;
   double k0, k1;
 };

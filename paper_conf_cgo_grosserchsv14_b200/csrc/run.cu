@@ -135,7 +135,6 @@ stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* 
         a.a_hi = l.a_hi;
         a.a_final = a_final;
         a.S0_lo = l.S0_lo;
-        a.S0_hi = l.S0_hi;
         a.row_off = l.row_off;
         a.W = p.W;
         a.k0 = d.coef[0];
