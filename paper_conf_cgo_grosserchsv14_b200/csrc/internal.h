@@ -112,6 +112,7 @@ stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* 
 int fast2d_variant(int kind, int dtype, int h, int w0, int w1);
 int fast2d_chunk_width(int variant);  // classical tile width w1 the kernel streams
 int fdtd_variant(int dtype, int h, int w0);
+int fdtd_ctas_per_sm();
 int fast3d_variant(int kind, int dtype, int h, int w0, int wy);
 int fast3d_tile(int variant, int* wy, int* wx);
 bool fast3d_variant_matches(int variant, int kind, int dtype, int h, int w0);

@@ -33,7 +33,11 @@ namespace fdtd {
 
 constexpr int C = 64;        // columns per chunk (= ring block)
 constexpr int RC = 4 * C;    // ring columns
-constexpr int RP = 4;        // threads per column (row parts, rows interleaved)
+#ifndef HEXS_FDTD_RP
+#define HEXS_FDTD_RP 4  // 2 (3 CTAs/SM) measured 228 -> 197 GUp/s
+#endif
+constexpr int RP = HEXS_FDTD_RP;  // threads per column (row parts, rows interleaved)
+constexpr int MINB = RP == 2 ? 3 : 2;  // resident CTAs per SM (shared memory: 3 fields x ring)
 constexpr int NT = RP * C;
 
 template <typename T>
@@ -57,7 +61,7 @@ __device__ __forceinline__ int64_t min64(int64_t a, int64_t b) { return a < b ? 
 
 // fields: 0 = ex, 1 = ey, 2 = hz (the order of FdtdArgs::f); statement k: 0 ey, 1 ex, 2 hz
 template <typename T>
-__global__ void __launch_bounds__(NT, 2) fdtd_kernel(const __grid_constant__ FdtdArgs g) {
+__global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ FdtdArgs g) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
   T* ring = reinterpret_cast<T*>(smem_raw);
   const int W = g.W, R = W + 2;  // smem rows: b in [-1, W] at b + 1
@@ -226,6 +230,8 @@ cudaError_t launch_t(const FdtdArgs& a, int grid, cudaStream_t s) {
 size_t fdtd_smem_bytes(int dtype, int W) {
   return dtype == 1 ? fdtd::smem_bytes<double>(W) : fdtd::smem_bytes<float>(W);
 }
+
+int fdtd_ctas_per_sm() { return fdtd::MINB; }
 
 cudaError_t launch_fdtd(int variant, const FdtdArgs& a, int grid, cudaStream_t s) {
   switch (variant) {

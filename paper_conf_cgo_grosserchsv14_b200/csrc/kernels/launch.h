@@ -71,6 +71,7 @@ struct FdtdArgs {
 };
 cudaError_t launch_fdtd(int variant, const FdtdArgs& a, int grid, cudaStream_t s);
 size_t fdtd_smem_bytes(int dtype, int W);
+int fdtd_ctas_per_sm();  // resident CTAs per SM the FDTD kernel is built for
 
 // 3D fast kernel (kernels/hex3d.cu): persistent CTAs run the classical tiles of every
 // hexagon of the launch as a tile-granular dependence wavefront, all levels of a tile in

@@ -177,11 +177,11 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
     if (d.kind == STENCIL_FDTD2D) {
       // 24 tau-levels = 8 full steps per tile (h+1 a multiple of 3, reading R14); w0 as
       // small as possible while every launch's hexagons (W = 2 w0 + 2 + h + h/2 rows) fit one
-      // wave of the FDTD kernel (2 CTAs per SM): a second, partial wave would double the
+      // wave of the FDTD kernel (fdtd_ctas_per_sm() CTAs per SM): a second, partial wave would double the
       // launch time (grid quantisation).  Best measured on B200: profiles/round1/.
       h = 11;
       w0 = 5;
-      const int64_t slots = 2 * (int64_t)device_sm_count();
+      const int64_t slots = (int64_t)fdtd_ctas_per_sm() * device_sm_count();
       auto Wof = [&](int w) { return (int64_t)2 * w + 2 + h + h / 2; };
       while (w0 < 12 && (d.ext[0] + Wof(w0) - 1) / Wof(w0) + 1 > slots) ++w0;
     } else if (d.dims == 2) {
