@@ -196,3 +196,33 @@ def test_full_size_fdtd():
     exp = oracle.fdtd(*[x.copy() for x in f], 500, nthreads=oracle.max_threads())
     for a, b, name in zip(got, exp, ("ex", "ey", "hz")):
         assert_bitexact(a, b, f"fdtd 8192^2 T=500 {name}")
+
+
+def test_slab_runner_nccl_single_rank():
+    """The multi-GPU slab path (paper_conf_cgo_grosserchsv14_b200/dist.py) on the GPU with a
+    one-rank NCCL process group: time blocks of D steps run back to back through the C-ABI
+    plans (including a remainder block) must reproduce the single-domain oracle bit-exactly."""
+    import os
+    import socket
+
+    import torch.distributed as tdist
+
+    from paper_conf_cgo_grosserchsv14_b200 import dist as hdist
+
+    sock = socket.socket()
+    sock.bind(("127.0.0.1", 0))
+    port = sock.getsockname()[1]
+    sock.close()
+    store = tdist.TCPStore("127.0.0.1", port, 1, True)
+    tdist.init_process_group("nccl", store=store, rank=0, world_size=1,
+                             device_id=torch.device("cuda", 0))
+    try:
+        for kind, ext, T, D in [("star2d5", (301, 517), 37, 16), ("star3d7", (40, 45, 68), 11, 4)]:
+            g = stencil_inputs.uniform(ext, seed=9)
+            runner = hdist.SlabRunner(kind, ext, T, D=D)
+            local = torch.from_numpy(np.ascontiguousarray(runner.scatter_view(g))).cuda()
+            runner.run(local)
+            torch.cuda.synchronize()
+            assert_bitexact(local.cpu().numpy(), oracle.run(kind, g, T), f"slab {kind} D={D}")
+    finally:
+        tdist.destroy_process_group()
