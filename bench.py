@@ -32,6 +32,9 @@ CONFIGS = {
     "fdtd2d": ("fdtd2d", (8192, 8192), 500, "fdtd-2D fp32, 8192x8192, T=500"),
     "heat3d": ("star3d7", (512, 512, 512), 128, "heat-3D 7-point fp32, 512^3, T=128"),
     "gradient3d": ("gradient3d", (512, 512, 512), 128, "gradient-3D fp32, 512^3, T=128"),
+    # the rest of the paper's Table 3 workload set, same grid sizes
+    "heat3d27": ("box3d27", (512, 512, 512), 128, "heat-3D 27-point fp32 (the paper's heat 3D), 512^3, T=128"),
+    "gradient2d": ("gradient2d", (8192, 8192), 512, "gradient-2D fp32, 8192x8192, T=512"),
 }
 METRIC = "GStencil-updates/s (fp32) at 1/2/4/8 B200 and % of time-tiled HBM roofline"
 

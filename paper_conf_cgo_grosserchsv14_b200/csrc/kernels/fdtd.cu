@@ -126,21 +126,7 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
     cp_async_commit();
   };
 
-  // per level (relative index a - a_lo): statement, rows [blo, bhi] clipped to the grid and
-  // the statement's domain (oracle/oracle.c: ey i >= 1; ex j >= 1; hz i < N0-1, j < N1-1),
-  // column range [jlo, jhi] of the statement
-  __shared__ int lv[kMaxH][5];
   const int nlev = g.a_hi - g.a_lo + 1;
-  if (tid < nlev) {
-    const int a = g.a_lo + tid;
-    const int st = (int)((g.tau0 + a) % 3);
-    const int64_t ilo = st == 0 ? 1 : 0, ihi = st == 2 ? N0 - 2 : N0 - 1;
-    lv[tid][0] = st;
-    lv[tid][1] = (int)max64(g.lo[a], ilo - i0);
-    lv[tid][2] = (int)min64(g.hi[a], ihi - i0);
-    lv[tid][3] = st == 1 ? 1 : 0;
-    lv[tid][4] = (int)(st == 2 ? N1 - 2 : N1 - 1);
-  }
   const int k_last = (int)((N1 - 1 + g.a_hi) / C);
   stage(0);
   stage(1);
@@ -153,10 +139,15 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
     stage(k + 3);          // next chunk's new block (ring slot of block k-1, written back)
     cp_async_wait<1>();    // every block but the newest has landed
     __syncthreads();
-    for (int l = 0; l < nlev; ++l) {
-      const int st = lv[l][0], blo = lv[l][1], bhi = lv[l][2];
-      const int j = k * C - (g.a_lo + l) + col;
-      if (j >= lv[l][3] && j <= lv[l][4]) {
+    int st = (int)((g.tau0 + g.a_lo) % 3);
+    for (int l = 0; l < nlev; ++l, st = st == 2 ? 0 : st + 1) {
+      // level parameters from the kernel arguments (constant bank), clipped to the grid and the
+      // statement's domain (oracle/oracle.c: ey i >= 1; ex j >= 1; hz i < N0-1, j < N1-1)
+      const int a = g.a_lo + l;
+      const int blo = max(g.lo[a], st == 0 ? (int)(1 - i0) : (int)(-i0));
+      const int bhi = min(g.hi[a], st == 2 ? (int)(N0 - 2 - i0) : (int)(N0 - 1 - i0));
+      const int j = k * C - a + col;
+      if (j >= (st == 1 ? 1 : 0) && j <= (st == 2 ? (int)N1 - 2 : (int)N1 - 1)) {
         // 32-bit shared-memory element offsets (one IADD per row step instead of 64-bit
         // pointer arithmetic); row b of field f at (f*R + b + 1) * RC + ring column
         const int cj = (j + C) & (RC - 1);
