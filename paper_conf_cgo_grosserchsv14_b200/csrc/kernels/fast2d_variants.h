@@ -22,5 +22,8 @@
   X(15, 0, float, K_BOX2D9, 2, 5, 4)             \
   X(16, 0, float, K_BOX2D9, 2, 7, 4)             \
   X(17, 0, float, K_BOX2D9, 4, 5, 4)             \
-  X(18, 0, float, K_BOX2D9, 3, 7, 8)
-#define HEXS_FAST2D_COUNT 19
+  X(18, 0, float, K_BOX2D9, 3, 7, 8)             \
+  X(19, 0, float, K_GRADIENT2D, 1, 3, 4)         \
+  X(20, 0, float, K_GRADIENT2D, 2, 3, 4)         \
+  X(21, 0, float, K_GRADIENT2D, 1, 1, 4)
+#define HEXS_FAST2D_COUNT 22

@@ -190,6 +190,8 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
       // instruction cache (ncu stall "no_instruction")
       h = 3; w0 = 7;
       if (d.kind == STENCIL_BOX2D9 && dtype == STENCIL_F32) h = 2;
+      // IEEE sqrt + div per point: only the smallest hexagon's body stays in the i-cache
+      if (d.kind == STENCIL_GRADIENT2D && dtype == STENCIL_F32) h = 1, w0 = 1;
     } else {
       h = 2; w0 = 7;  // Table 4 setup
     }
