@@ -25,5 +25,9 @@
   X(18, 0, float, K_BOX2D9, 3, 7, 8)             \
   X(19, 0, float, K_GRADIENT2D, 1, 3, 4)         \
   X(20, 0, float, K_GRADIENT2D, 2, 3, 4)         \
-  X(21, 0, float, K_GRADIENT2D, 1, 1, 4)
-#define HEXS_FAST2D_COUNT 22
+  X(21, 0, float, K_GRADIENT2D, 1, 1, 4)         \
+  X(22, 0, float, K_STAR2D5, 2, 7, 4)            \
+  X(23, 0, float, K_STAR2D5, 2, 9, 4)            \
+  X(24, 0, float, K_BOX2D9, 2, 9, 4)             \
+  X(25, 0, float, K_STAR2D5, 3, 9, 4)
+#define HEXS_FAST2D_COUNT 26
