@@ -60,13 +60,13 @@ constexpr int NQ = NX / 4;     // column quads: one 8-lane group
 constexpr int SIGMA = 4;       // x skew per level
 // Carry areas (the predecessor tiles' values): the carry-column quad (main-frame m = -4 .. -1)
 // and the edge column (m = -5, element 3 of its quad) in areas of 16-B lines, and 2 carry lines.
-// Each TMA box starts a few lines early (SC, SL) and rows are padded to 8-chunk multiples, so
+// The carry-quad and edge boxes start SC lines early and their rows are padded to 8-chunk multiples, so
 // that lane 0's carry quad lands in the one 16-B bank slot its 8-lane group leaves free in the
 // same LDS.128 (conflict-free; a TMA destination itself must stay 128-B aligned).
 // (fp32 bank geometry; the fp64 variants keep the dense 2-line / NY+2-line areas)
 template <typename T> constexpr int SC = sizeof(T) == 4 ? 5 : 0;  // line shift of the carry boxes
-template <typename T> constexpr int SL = sizeof(T) == 4 ? 6 : 0;  // line shift of the carry-line box
-template <typename T> constexpr int LR = sizeof(T) == 4 ? 8 : 2;  // lines per row, carry-line area
+template <typename T> constexpr int SL = 0;  // line shift of the carry-line box
+template <typename T> constexpr int LR = 2;  // lines per row, carry-line area (its 2 of NY+2 lines may conflict)
 template <typename T> constexpr int CLP = sizeof(T) == 4 ? 8 : 2; // extra lines per row, carry areas
 
 // Hexagon of a radius-1 single-statement stencil (delta0 = delta1 = 1): rows b of level a
