@@ -237,6 +237,27 @@ __device__ __forceinline__ void named_barrier_sync(int id, int nthreads) {
   asm volatile("bar.sync %0, %1;" ::"r"(id), "r"(nthreads) : "memory");
 }
 
+// Optional event trace (debug builds: -DHEXS_F3_TRACE): CTAs 0..7 record (type, tile, level,
+// clock64) for the producer lane and compute thread 0; tools/f3_trace.py prints the timeline.
+#ifdef HEXS_F3_TRACE
+constexpr int kTrCtas = 8, kTrEv = 8192;
+__device__ unsigned long long g_f3_tr[kTrCtas][kTrEv];
+__device__ int g_f3_trn[kTrCtas];
+__device__ __forceinline__ void f3_trace(int type, int tile, int level) {
+  if (blockIdx.x < kTrCtas) {
+    const int i = atomicAdd(&g_f3_trn[blockIdx.x], 1);
+    if (i < kTrEv)
+      g_f3_tr[blockIdx.x][i] = ((unsigned long long)type << 60) | ((unsigned long long)(tile & 0xFFFF) << 44) |
+                               ((unsigned long long)(level & 0xFF) << 36) | ((unsigned long long)clock64() & 0xFFFFFFFFFull);
+  }
+}
+#define F3_TR(type, tile, level) f3_trace(type, tile, level)
+#else
+#define F3_TR(type, tile, level) \
+  do {                            \
+  } while (0)
+#endif
+
 template <int... As, typename F>
 __device__ __forceinline__ void for_levels(F&& f, std::integer_sequence<int, As...>) {
   (f(std::integral_constant<int, As>{}), ...);
@@ -385,7 +406,7 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
     // fill(a_lo + 1) is issued).
     if (tid == NC) {
       uint32_t fills[2] = {0u, 0u};
-      int slot = 0;
+      int slot = 0, ptile = 0;
       while (true) {
         long long* it = item_s[slot];
         decode((int64_t)atomicAdd(g.counter, 1ull), it);
@@ -398,6 +419,7 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
         const int64_t base = (it[0] - g.S0_lo) * n1 * n2;
         for (int a = a_lo; a <= a_hi; ++a) {
           const int b = a & 1;
+          F3_TR(1, ptile, a);
           if (fills[b] > 0) mbar_wait_parity(&empty[b], (fills[b] - 1) & 1u);
           F3_TM(0);
           fence_proxy_async_smem();
@@ -405,12 +427,14 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
             issue_first(it, a);
           } else {
             if (a == a_lo + 1) {  // predecessors complete: their carries are in global memory
+              F3_TR(3, ptile, a);
               const int* f = g.flags + base;
               if (it[1] > 0)
                 while (ld_acquire(f + (it[1] - 1) * n2 + it[2]) == 0) __nanosleep(64);
               if (it[2] > 0)
                 while (ld_acquire(f + it[1] * n2 + it[2] - 1) == 0) __nanosleep(64);
               fence_proxy_async_global();
+              F3_TR(4, ptile, a);
               F3_TM(2);
             }
             mbar_arrive_expect_tx(&full[b], LY::CARRY_BYTES + (a <= H + 1 ? in_bytes(a) : 0u));
@@ -418,8 +442,10 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
             issue_carries(it, a);
           }
           ++fills[b];
+          F3_TR(2, ptile, a);
           F3_TM(4);
         }
+        ++ptile;
         slot ^= 1;
       }
     }
@@ -430,7 +456,7 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
   uint32_t ph = 0u;  // parity bit per buffer
   const Coef<T> cf{(T)g.k0, (T)g.k1};
   const int lane = tid & 31;
-  int slot = 0;
+  int slot = 0, ctile = 0;
   while (true) {
     {
       const int b0 = a_lo & 1;  // the tile's first fill publishes its item
@@ -463,10 +489,12 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
           constexpr int N = (HI - LO + 1 + ZS - 1) / ZS;
           const int R0 = zpart == 0 ? LO : HI - N + 1;
           const int dR = R0 - LO;
+          if (tid == 0) F3_TR(5, ctile, A);
           if (A != a_lo) mbar_wait_parity(&full[b], (ph >> b) & 1u);
           ph ^= 1u << b;
           F3_TM(0);
           named_barrier_sync(1, NC);  // level A-1's buffer writes visible to every compute warp
+          if (tid == 0) F3_TR(6, ctile, A);
           F3_TM(1);
 
           // ---- compute level A: line y = Y0 - A + ly, x = X0 - 4A + 4q + j, rows [LO, HI]
@@ -602,12 +630,15 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
           fence_proxy_async_smem();
           __syncwarp();
           if (lane == 0) mbar_arrive(&empty[b]);
+          if (tid == 0) F3_TR(7, ctile, A);
           F3_TM(3);
         },
         std::make_integer_sequence<int, L>{});
     named_barrier_sync(1, NC);  // every compute thread's stores of the tile are issued
     F3_TM(1);
     if (tid == 0) st_release(my_flag, 1);
+    if (tid == 0) F3_TR(8, ctile, 0);
+    ++ctile;
     slot ^= 1;
   }
 }
@@ -686,6 +717,17 @@ using S3 = Sel3<HEXS_F3_VARIANT>;
 cudaError_t HEXS_F3_CAT(launch_fast3d_v, HEXS_F3_VARIANT)(const Fast3DArgs& a, cudaStream_t s) {
   return fast3d::launch_t<S3::T, S3::KIND, S3::H, S3::W0, S3::NY, S3::MINB, S3::ZS>(a, s);
 }
+#ifdef HEXS_F3_TRACE
+extern "C" int HEXS_F3_CAT(hexs_f3_trace_v, HEXS_F3_VARIANT)(unsigned long long* host, int* counts, int reset) {
+  if (cudaMemcpyFromSymbol(host, fast3d::g_f3_tr, sizeof(fast3d::g_f3_tr)) != cudaSuccess) return -1;
+  if (cudaMemcpyFromSymbol(counts, fast3d::g_f3_trn, sizeof(fast3d::g_f3_trn)) != cudaSuccess) return -1;
+  if (reset) {
+    static int zero[fast3d::kTrCtas];
+    cudaMemcpyToSymbol(fast3d::g_f3_trn, zero, sizeof(zero));
+  }
+  return 0;
+}
+#endif
 #ifdef HEXS_F3_TIMING
 extern "C" int HEXS_F3_CAT(hexs_f3_timing_v, HEXS_F3_VARIANT)(unsigned long long* host, int reset) {
   if (cudaMemcpyFromSymbol(host, fast3d::g_f3_tm, sizeof(fast3d::g_f3_tm)) != cudaSuccess) return -1;
