@@ -194,6 +194,9 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
       if (d.kind == STENCIL_GRADIENT2D && dtype == STENCIL_F32) h = 1, w0 = 1;
     } else {
       h = 2; w0 = 7;  // Table 4 setup
+      // the 7-point star: one more level pair per tile amortises the per-tile fills and flags
+      // (measured 527 -> 550 GUp/s; profiles/round1/tile_sweep_heat3d.txt)
+      if (d.kind == STENCIL_STAR3D7 && dtype == STENCIL_F32) h = 3;
     }
   }
   if (h < 0 || w0 < 0) return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_plan: negative tile parameter");
