@@ -9,8 +9,8 @@
 //     j in [kC - a, kC - a + C - 1] -- the classical tile of eq. (14) with w1 = C, u = a --
 //     and the chunks run sequentially inside the CTA, as the paper's S1 loop does;
 //   * all three fields of the hexagon's rows (plus the halo rows -1 and W the statements
-//     read) live in a shared-memory RING of 4 blocks of C columns (column j at ring index
-//     (j + C) mod 4C), so the columns a chunk shares with its predecessor (the skewed
+//     read) live in a shared-memory RING of NB blocks of C columns (column j at ring index
+//     (j + C) mod NB*C), so the columns a chunk shares with its predecessor (the skewed
 //     overlap) are reused on chip -- the inter-tile reuse of Sec. 4.2.2;
 //   * the block a chunk will need next is prefetched one chunk ahead with 16-B cp.async
 //     (LDGSTS, every address 16-B aligned -- the aligned loads of Sec. 4.2.3), so no warp
@@ -32,12 +32,19 @@ namespace hexs {
 namespace fdtd {
 
 constexpr int C = 64;        // columns per chunk (= ring block)
-constexpr int RC = 4 * C;    // ring columns
+#ifndef HEXS_FDTD_RING
+#define HEXS_FDTD_RING 4  // 3 (3 CTAs/SM, one-chunk prefetch) measured 226 -> 192 GUp/s
+#endif
+// Ring of NB blocks of C columns: 4 (prefetch two chunks ahead, 2 CTAs/SM) or 3 (one chunk
+// ahead; 3 CTAs/SM fit the shared memory).  Ring column of grid column j: (j + C) mod RC.
+constexpr int NB = HEXS_FDTD_RING;
+constexpr int RC = NB * C;    // ring columns
+__device__ __forceinline__ int ring_col(int j) { return (j + C) % RC; }  // j >= -C
 #ifndef HEXS_FDTD_RP
 #define HEXS_FDTD_RP 4  // 2 (3 CTAs/SM) measured 228 -> 197 GUp/s
 #endif
 constexpr int RP = HEXS_FDTD_RP;  // threads per column (row parts, rows interleaved)
-constexpr int MINB = RP == 2 ? 3 : 2;  // resident CTAs per SM (shared memory: 3 fields x ring)
+constexpr int MINB = (RP == 2 || NB == 3) ? 3 : 2;  // resident CTAs per SM (shared memory: 3 fields x ring)
 constexpr int NT = RP * C;
 
 template <typename T>
@@ -116,7 +123,7 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
   auto stage = [&](int blk) {
     const int j = (blk - 1) * C + sc * CH;
     const bool jok = j >= 0 && j < N1;
-    const int cj = (j + C) & (RC - 1);
+    const int cj = ring_col(j);
 #pragma unroll
     for (int u = 0; u < MAXU; ++u) {
       if (soff[u] < 0) continue;
@@ -128,15 +135,13 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
 
   const int nlev = g.a_hi - g.a_lo + 1;
   const int k_last = (int)((N1 - 1 + g.a_hi) / C);
-  stage(0);
-  stage(1);
-  stage(2);
+  for (int blk = 0; blk < NB - 1; ++blk) stage(blk);
   const int col = tid & (C - 1), rpar = tid / C;  // column, row part
   T* const rex = ring + (size_t)(0 * R + 1) * RC;  // row b of a field at r.. + b * RC + ring column
   T* const rey = ring + (size_t)(1 * R + 1) * RC;
   T* const rhz = ring + (size_t)(2 * R + 1) * RC;
   for (int k = 0; k <= k_last; ++k) {
-    stage(k + 3);          // next chunk's new block (ring slot of block k-1, written back)
+    stage(k + NB - 1);     // a later chunk's new block (ring slot of block k-1, written back)
     cp_async_wait<1>();    // every block but the newest has landed
     __syncthreads();
     int st = (int)((g.tau0 + g.a_lo) % 3);
@@ -150,7 +155,7 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
       if (j >= (st == 1 ? 1 : 0) && j <= (st == 2 ? (int)N1 - 2 : (int)N1 - 1)) {
         // 32-bit shared-memory element offsets (one IADD per row step instead of 64-bit
         // pointer arithmetic); row b of field f at (f*R + b + 1) * RC + ring column
-        const int cj = (j + C) & (RC - 1);
+        const int cj = ring_col(j);
         const int b0 = blo + rpar;
         int o = (b0 + 1) * RC + cj;  // row b0 of a field, relative to its first row
         constexpr int STEP = RP * RC;
@@ -162,7 +167,7 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
             *pe = fdtd_ey<T>(*pe, ph[0], ph[-RC], cf);
           }
         } else if (st == 1) {  // ex[i][j] -= ce * (hz[i][j] - hz[i][j-1])
-          const int dm = ((j - 1 + C) & (RC - 1)) - cj;  // column j-1 relative to j in the ring
+          const int dm = ring_col(j - 1) - cj;  // column j-1 relative to j in the ring
 #pragma unroll 4
           for (int b = b0; b <= bhi; b += RP, o += STEP) {
             T* px = ring + o;
@@ -170,7 +175,7 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
             *px = fdtd_ex<T>(*px, ph[0], ph[dm], cf);
           }
         } else {  // hz[i][j] -= ch * (((ex[i][j+1] - ex[i][j]) + ey[i+1][j]) - ey[i][j])
-          const int dp = ((j + 1 + C) & (RC - 1)) - cj;  // column j+1 relative to j in the ring
+          const int dp = ring_col(j + 1) - cj;  // column j+1 relative to j in the ring
 #pragma unroll 4
           for (int b = b0; b <= bhi; b += RP, o += STEP) {
             T* ph = ring + 2 * R * RC + o;
@@ -188,7 +193,7 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
     const int whi = (k == k_last) ? (int)N1 - 1 : (k + 1) * C - g.a_hi - 1;
     for (int j = k * C - g.a_hi + col; j <= whi; j += C) {
       if (j < wlo) continue;
-      const int cj = (j + C) & (RC - 1);
+      const int cj = ring_col(j);
 #pragma unroll
       for (int f = 0; f < 3; ++f) {
         const int b0 = mlo[f] + rpar;
