@@ -47,6 +47,9 @@
 #ifndef HEXS_F3_UNROLL
 #define HEXS_F3_UNROLL 1  // 0: rolled star sweeps (smaller code; measured equal or slower)
 #endif
+#ifndef HEXS_F3_LEAD
+#define HEXS_F3_LEAD 1  // window rows loaded ahead of the shuffled row (2, 3 measured 544, 545 vs 551)
+#endif
 #ifndef HEXS_F3_VARIANT
 #error "hex3d.cu is compiled once per fast3d variant: -DHEXS_F3_VARIANT=<id>"
 #endif
@@ -570,19 +573,20 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
             // short per-point expression: the whole sweep unrolled and software-pipelined
             // (loads of row i+3, edges of row i+2, arithmetic of row i+1)
             // row i+1 needs its edges before step(i); rows' shuffles run one row earlier
+            // HEXS_F3_LEAD rows of loads in flight ahead of the row being shuffled
+            constexpr int LD = HEXS_F3_LEAD;
             Win<T> w[N + 2];
-            load_win<T, E27>(w[0], Pr, q, eo);
-            adv();
-            load_win<T, E27>(w[1], Pr, q, eo);
-            adv();
-            load_win<T, E27>(w[2], Pr, q, eo);
-            adv();
+#pragma unroll
+            for (int r = 0; r < 3 + LD - 1 && r < N + 2; ++r) {
+              load_win<T, E27>(w[r], Pr, q, eo);
+              adv();
+            }
             Edge<T> e1 = edges_shfl(w[1]);
             Edge<T> e2 = edges_shfl(w[2]);
 #pragma unroll
             for (int i = 0; i < N; ++i) {
-              if (i + 3 < N + 2) {
-                load_win<T, E27>(w[i + 3], Pr, q, eo);
+              if (i + 3 + LD - 1 < N + 2) {
+                load_win<T, E27>(w[i + 3 + LD - 1], Pr, q, eo);
                 adv();
               }
               edges_sel(w[i + 1], e1, q);
