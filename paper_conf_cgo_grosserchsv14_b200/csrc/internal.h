@@ -94,6 +94,15 @@ struct Plan {
   // profiling: event pairs around each launch for up to prof_runs runs
   int prof_runs = 0, prof_used = 0;
   std::vector<void*> prof_events;  // cudaEvent_t, 2 per launch per run
+  // CUDA graphs of whole runs (the launch sequence is fixed by the plan): keyed by the field,
+  // workspace pointers; replayed on the caller's stream (a run is launch-bound on small grids)
+  struct GraphEntry {
+    std::vector<const void*> key;
+    void* exec = nullptr;  // cudaGraphExec_t
+  };
+  std::vector<GraphEntry> graphs;
+  int eager_runs = 0;      // runs executed eagerly (the first one sets kernel attributes)
+  void* capture_stream = nullptr;
   ~Plan();
 };
 
