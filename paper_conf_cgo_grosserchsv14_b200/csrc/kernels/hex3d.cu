@@ -108,6 +108,7 @@ template <typename T, int Q, int NY> struct Lay {
 
 struct Maps {
   CUtensorMap main[2];   // box {NXP, NY, Q}
+  CUtensorMap main0[2];  // box {NXP, NY, W0+3}: the rows level 0 reads (full-time tiles)
   CUtensorMap lines[2];  // box {NXP, LR, Q}
   CUtensorMap carry[2];  // box {4, NY+8, Q} (carry quads and edge columns)
   CUtensorMap in2[2];    // box {NXP, NY, 2}
@@ -350,8 +351,15 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
     const int b = a & 1, par = (int)((g.tau0 + a) & 1);
     const int z0 = (int)(i0 - 1), xo = X0 - SIGMA * a, yo = Y0 - a;
     T* B = buf_of(b);
-    mbar_arrive_expect_tx(&full[b], LY::FIRST_BYTES);
-    tma_3d(B, &mp.main[par], xo + 4, yo + 1, z0, &full[b]);
+    if (a == 0) {  // only the rows level 0 reads: [lo(0)-1, hi(0)+1] (W0+3 of the Q rows)
+      constexpr uint32_t FB0 =
+          (uint32_t)(((HX::hi(0) - HX::lo(0) + 3) * LY::MAIN + Q * (LY::LINES + 2 * LY::CARRY)) * sizeof(T));
+      mbar_arrive_expect_tx(&full[b], FB0);
+      tma_3d(B + HX::lo(0) * LY::MAIN, &mp.main0[par], xo + 4, yo + 1, (int)(i0 + HX::lo(0) - 1), &full[b]);
+    } else {
+      mbar_arrive_expect_tx(&full[b], LY::FIRST_BYTES);
+      tma_3d(B, &mp.main[par], xo + 4, yo + 1, z0, &full[b]);
+    }
     tma_3d(B + LY::LINES_OFF, &mp.lines[par], xo + 4, yo - 1 - SL<T>, z0, &full[b]);
     tma_3d(B + LY::CARRY_OFF, &mp.carry[par], xo, yo - 1 - SC<T>, z0, &full[b]);
     tma_3d(B + LY::EDGE_OFF, &mp.carry[par], xo - 4, yo - 1 - SC<T>, z0, &full[b]);
@@ -692,7 +700,8 @@ cudaError_t launch_t(const Fast3DArgs& a, cudaStream_t s) {
   Maps m;
   const uint32_t Q = (uint32_t)a.Q, ny = (uint32_t)NY;
   for (int b = 0; b < 2; ++b) {
-    if (!encode<T>(&m.main[b], a.buf[b], a, NXP, ny, Q) || !encode<T>(&m.lines[b], a.buf[b], a, NXP, LR<T>, Q) ||
+    if (!encode<T>(&m.main[b], a.buf[b], a, NXP, ny, Q) ||
+        !encode<T>(&m.main0[b], a.buf[b], a, NXP, ny, (uint32_t)(W0 + 3)) || !encode<T>(&m.lines[b], a.buf[b], a, NXP, LR<T>, Q) ||
         !encode<T>(&m.carry[b], a.buf[b], a, 4, ny + CLP<T>, Q) || !encode<T>(&m.in2[b], a.buf[b], a, NXP, ny, 2) ||
         !encode<T>(&m.in1[b], a.buf[b], a, NXP, ny, 1))
       return cudaErrorInvalidValue;
