@@ -4,15 +4,17 @@
 // hexagon shape is a compile-time parameter (every level's row range is unrolled, "constraint-based unrolling"); each id is
 // compiled from hex3d.cu with -DHEXS_F3_VARIANT=id into its own object (parallel build).
 // (2, 7) is the default 3D tile (Table 4's h = 2); the star3d7 fp32
-// shapes serve the tile sweep and the tests; a
+// shapes serve the tile sweep and the tests; the long gradient / 27-point expressions split each
+// column's rows over 2 threads (ZS = 2: 16 compute warps hide their latency; gradient 232 -> 321
+// GUp/s); a
 // tile whose classical width w[0] is set selects the variant with NY = w[0].  Other (h, w0) run the generic hybrid kernel.
 #pragma once
 #define HEXS_FAST3D_VARIANTS(X)                 \
   X(0, 0, float, K_STAR3D7, 2, 7, 32, 1, 1)     \
   X(1, 1, double, K_STAR3D7, 2, 7, 16, 1, 1)    \
-  X(2, 0, float, K_GRADIENT3D, 2, 7, 32, 1, 1)  \
+  X(2, 0, float, K_GRADIENT3D, 2, 7, 32, 1, 2)  \
   X(3, 1, double, K_GRADIENT3D, 2, 7, 16, 1, 1) \
-  X(4, 0, float, K_BOX3D27, 2, 7, 32, 1, 1)     \
+  X(4, 0, float, K_BOX3D27, 2, 7, 32, 1, 2)     \
   X(5, 1, double, K_BOX3D27, 2, 7, 16, 1, 1)    \
   X(6, 0, float, K_STAR3D7, 1, 3, 16, 2, 1)     \
   X(7, 0, float, K_STAR3D7, 3, 2, 16, 2, 1)     \
