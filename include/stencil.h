@@ -123,7 +123,11 @@ stencil_status stencil_plan_set_workspace(stencil_plan_t plan, void *dev_ptr, si
  *   T_steps   must equal the plan's (STENCIL_E_INVALID otherwise); 0 copies in to out.
  *   stream    cudaStream_t as void*; all work is enqueued on it (asynchronous).
  * Per launch-table entry (T, p) one phase kernel is launched (host loop over T and the
- * two phases). */
+ * two phases).  From the second call with the same in/out/workspace
+ * pointers (and no profiling requested) the plan replays a CUDA graph of the whole launch
+ * sequence, captured once on a private stream and launched on `stream` (same results,
+ * less launch overhead; environment HEXS_NO_GRAPH=1 keeps every run eager).  The graphs
+ * are released with the plan. */
 stencil_status stencil_run(stencil_plan_t plan, const void *const *in, void *const *out,
                            int64_t T_steps, void *stream);
 
