@@ -49,6 +49,7 @@ class Statement:
     reads: Tuple[Tuple[str, Tuple[int, ...]], ...]
     lo: Tuple[int, ...]  # domain lower bound per spatial dim, relative to 0
     hi: Tuple[int, ...]  # domain upper bound per spatial dim, relative to N (exclusive): N + hi
+    versions: Tuple[int, ...] = ()  # time-expanded layout only: read i reads A[t + versions[i]]
 
 
 @dataclass(frozen=True)
@@ -56,6 +57,7 @@ class Program:
     dims: int
     statements: Tuple[Statement, ...]
     pingpong: bool
+    expanded: bool = False  # time-expanded arrays A[t][s]: no location is ever reused
 
 
 def single_statement(offsets: Sequence[Tuple[int, ...]]) -> Program:
@@ -91,6 +93,17 @@ FDTD2D = Program(
 )
 
 
+def expanded_program(reads: Sequence[Tuple[int, Tuple[int, ...]]], lo: Sequence[int],
+                     hi: Sequence[int]) -> Program:
+    """A[t][s] = f(A[t + dt][s + ds] for (dt, ds) in reads) with a time-expanded array (every
+    version has its own memory), e.g. the example of Sec. 3.3.2,
+    A[t][i] = f(A[t-2][i-2], A[t-1][i+2]) (PAPER.md:346-350)."""
+    dims = len(reads[0][1])
+    st = Statement("A", tuple(("A", tuple(o)) for _, o in reads), tuple(lo), tuple(hi),
+                   tuple(dt for dt, _ in reads))
+    return Program(dims, (st,), False, True)
+
+
 def instances(prog: Program, N: Sequence[int], steps: int):
     """Statement instances in the ORIGINAL program order, as (tau, s) with the canonical
     time tau = k*t + i (Sec. 3.2)."""
@@ -102,32 +115,54 @@ def instances(prog: Program, N: Sequence[int], steps: int):
                 yield k * t + i, s, st, t
 
 
-def dependences(prog: Program, N: Sequence[int], steps: int) -> List[Tuple[Tuple, Tuple]]:
+def dependences(prog: Program, N: Sequence[int], steps: int, typed: bool = False) -> List[Tuple]:
     """All memory-based dependences (RAW, WAR, WAW) between instances, by simulating the
     original execution order over the actual memory locations (Sec. 3.1: 'This dependence
     relation can be computed from the iteration domain, the access relation and a
     description of the original execution order').  Returns pairs
-    (source instance, sink instance), instances as (tau, s)."""
+    (source instance, sink instance), instances as (tau, s); with typed=True triples
+    (kind, source, sink), kind in {"RAW", "WAR", "WAW"}.
+
+    Memory locations: ping-pong (Fig. 1) -- step t reads A[t%2] and
+    writes A[(t+1)%2]; in place (FDTD) -- one copy per array; time-expanded -- step t
+    writes A[t] and reads A[t + dt] (no location reused)."""
     last_write: Dict[Tuple, Tuple] = {}
     readers: Dict[Tuple, List[Tuple]] = {}
     deps = []
+
+    def add(kind, src, snk):
+        deps.append((kind, src, snk) if typed else (src, snk))
+
     for tau, s, st, t in instances(prog, N, steps):
         me = (tau, s)
-        for arr, o in st.reads:
+        for i, (arr, o) in enumerate(st.reads):
             loc_s = tuple(s[d] + o[d] for d in range(prog.dims))
-            loc = (arr, t % 2 if prog.pingpong else 0, loc_s)
+            if prog.expanded:
+                slot = t + st.versions[i]
+            else:
+                slot = t % 2 if prog.pingpong else 0
+            loc = (arr, slot, loc_s)
             if loc in last_write:
-                deps.append((last_write[loc], me))  # RAW
+                add("RAW", last_write[loc], me)
             readers.setdefault(loc, []).append(me)
-        wloc = (st.write, (t + 1) % 2 if prog.pingpong else 0, tuple(s))
+        wslot = t if prog.expanded else ((t + 1) % 2 if prog.pingpong else 0)
+        wloc = (st.write, wslot, tuple(s))
         if wloc in last_write:
-            deps.append((last_write[wloc], me))  # WAW
+            add("WAW", last_write[wloc], me)
         for r in readers.get(wloc, []):
             if r != me:
-                deps.append((r, me))  # WAR
+                add("WAR", r, me)
         readers[wloc] = []
         last_write[wloc] = me
     return deps
+
+
+def typed_distance_vectors(deps) -> Dict[str, set]:
+    """{kind: distance vectors} of typed dependences (dependences(..., typed=True))."""
+    out: Dict[str, set] = {"RAW": set(), "WAR": set(), "WAW": set()}
+    for kind, a, b in deps:
+        out[kind].add(tuple([b[0] - a[0]] + [b[1][d] - a[1][d] for d in range(len(a[1]))]))
+    return out
 
 
 def distance_vectors(deps) -> set:

@@ -168,3 +168,59 @@ def test_larger_skew_and_translation_stay_valid(offsets):
     r = S.check_schedule(prog, N, 7, S.Hex(Fr(1), Fr(1), 1, 1), [Fr(1), Fr(4)], [3, 8],
                          trans=[0, 1])
     assert r["coverage"] == r["order"] == r["same_phase"] == r["same_step"] == 0, r
+
+
+# ---- pins of the dependence simulator itself (oracle/schedule.py::dependences) ----------
+# The sets below are fixed by the paper's programs and the memory layout, derived by hand
+# (no call into the code under test): a plausible slip in the simulator (a dropped WAR or
+# WAW edge, a wrong parity slot, a reversed offset) changes one of them.
+
+def test_dependences_fig1_pingpong_exact_set():
+    """Fig. 1 (PAPER.md:142-148): A[(t+1)%2][i][j] = f(A[t%2][i+-1][j], A[t%2][i][j+-1],
+    A[t%2][i][j]).  RAW: the value read at offset o was written one step earlier at s+o:
+    (1, -o).  WAR: the location A[t%2][s+o] read at step t is overwritten at step t+1 by the
+    instance at s+o: (1, o).  WAW: A[(t+1)%2][s] is rewritten at step t+2: (2, 0)."""
+    prog = S.single_statement(S.STAR2D5)
+    typed = S.typed_distance_vectors(S.dependences(prog, (7, 8), 4, typed=True))
+    star = {(1, 0, 0), (1, 1, 0), (1, -1, 0), (1, 0, 1), (1, 0, -1)}
+    assert typed["RAW"] == star
+    assert typed["WAR"] == star
+    assert typed["WAW"] == {(2, 0, 0)}
+    assert S.distance_vectors(S.dependences(prog, (7, 8), 4)) == star | {(2, 0, 0)}
+
+
+def test_dependences_one_sided_stencil_separates_raw_from_war():
+    """A one-sided ping-pong stencil A'[s] = f(A[s], A[s+1]): RAW distances (1, -o) =
+    {(1,0), (1,-1)}, WAR distances (1, +o) = {(1,0), (1,1)}, WAW (2,0).  Dropping the WAR
+    edges loses (1, 1); dropping WAW loses (2, 0); swapping RAW/WAR flips the signs."""
+    prog = S.single_statement([(0,), (1,)])
+    typed = S.typed_distance_vectors(S.dependences(prog, (12,), 5, typed=True))
+    assert typed == {"RAW": {(1, 0), (1, -1)}, "WAR": {(1, 0), (1, 1)}, "WAW": {(2, 0)}}
+    assert S.distance_vectors(S.dependences(prog, (12,), 5)) == {(1, 0), (1, -1), (1, 1), (2, 0)}
+    # the cone these span: delta0 = 1 (from (1, 1), a WAR edge), delta1 = 1 (RAW (1, -1))
+    assert S.slopes(S.distance_vectors(S.dependences(prog, (12,), 5))) == (1, 1)
+
+
+def test_dependences_paper_example_through_simulator():
+    """The example of Sec. 3.3.2, A[t][i] = f(A[t-2][i-2], A[t-1][i+2]) with a time-expanded
+    array, has exactly the distance vectors {(1,-2); (2,2)}: RAW only,
+    since no location is reused.  Fed through the memory simulator, then Fig. 3's slopes."""
+    prog = S.expanded_program([(-2, (-2,)), (-1, (2,))], lo=(2,), hi=(-2,))
+    typed = S.typed_distance_vectors(S.dependences(prog, (16,), 7, typed=True))
+    assert typed == {"RAW": {(1, -2), (2, 2)}, "WAR": set(), "WAW": set()}
+    assert S.slopes(S.distance_vectors(S.dependences(prog, (16,), 7))) == (1, 2)
+
+
+def test_dependences_fdtd_exact_sets():
+    """FDTD-2D in place with tau = 3t+k (ey k=0, ex k=1, hz k=2; Sec. 3.2),
+    derived by hand from the three statements (reading R9):
+      RAW  ey<-hz(t-1): (1,0,0), (1,1,0); ex<-hz(t-1): (2,0,0), (2,0,1);
+           hz<-ex(t): (1,0,-1), (1,0,0); hz<-ey(t): (2,-1,0), (2,0,0); self: (3,0,0)
+      WAR  hz(t) overwrites what ey(t) read: (2,0,0), (2,-1,0); what ex(t) read: (1,0,0),
+           (1,0,-1); ex(t+1) overwrites what hz(t) read: (2,0,1), (2,0,0); ey(t+1): (1,1,0),
+           (1,0,0)
+      WAW  every field once per step: (3,0,0)"""
+    typed = S.typed_distance_vectors(S.dependences(S.FDTD2D, (7, 8), 4, typed=True))
+    assert typed["RAW"] == {(1, 0, 0), (1, 1, 0), (2, 0, 0), (2, 0, 1), (1, 0, -1), (2, -1, 0), (3, 0, 0)}
+    assert typed["WAR"] == {(2, 0, 0), (2, -1, 0), (1, 0, 0), (1, 0, -1), (2, 0, 1), (1, 1, 0)}
+    assert typed["WAW"] == {(3, 0, 0)}
