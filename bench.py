@@ -206,26 +206,54 @@ def make_inputs(kind, ext, seed=0):
     return [stencil_inputs.uniform(ext, seed=seed)]
 
 
+def _keep_heap_pages():
+    """glibc: serve large mallocs from the heap and never trim it, so the oracle's per-call
+    buffers reuse already-faulted pages instead of fresh mmap'd ones (page faults would
+    otherwise dominate a short call).  Does not touch the oracle's arithmetic."""
+    try:
+        import ctypes
+
+        libc = ctypes.CDLL("libc.so.6")
+        M_TRIM_THRESHOLD, M_MMAP_THRESHOLD = -1, -3
+        libc.mallopt(M_MMAP_THRESHOLD, 1 << 30)  # max allowed by glibc: 32 MiB..1 GiB blocks from the heap
+        libc.mallopt(M_TRIM_THRESHOLD, 1 << 62)
+    except OSError:
+        pass
+
+
 def run_reference(args, cfg):
+    """The CPU oracle as it stands, on the host cores, on this arm's config / metric.  Each
+    step is a bounded sample of the workload: the full grid for `steps_per` of its time steps
+    (about a second of work).  oracle.run copies the grid in and out on every call; that fixed
+    per-call cost is measured with 0-step calls and subtracted, so the number is the oracle's
+    time-stepping rate (what cpu_baseline reports), not its argument marshalling."""
     kind, ext, T, cname = CONFIGS[cfg]
     rank = int(os.environ.get("RANK", "0"))
     if rank != 0:
         return
+    _keep_heap_pages()
     import oracle
 
     nthreads = oracle.max_threads()
     fields = make_inputs(kind, ext)
-    # bounded sample per step: the workload's grid for a few of its time steps
-    steps_per = 4 if kind != "fdtd2d" else 2
-    times = []
-    for i in range(args.warmup + args.steps):
+
+    def call(n):
         t0 = time.perf_counter()
         if kind == "fdtd2d":
-            oracle.fdtd(*fields, steps_per, nthreads=nthreads)
+            oracle.fdtd(*fields, n, nthreads=nthreads)
         else:
-            oracle.run(kind, fields[0], steps_per, nthreads=nthreads)
+            oracle.run(kind, fields[0], n, nthreads=nthreads)
+        return time.perf_counter() - t0
+
+    call(1)  # first touch of the heap pages and thread start
+    overhead = float(np.median([call(0) for _ in range(3)]))
+    per = max(1e-6, call(4) - overhead) / 4
+    steps_per = int(max(2, min(T, round(1.0 / per))))
+    times = []
+    for i in range(args.warmup + args.steps):
+        dt = call(steps_per) - overhead
         if i >= args.warmup:
-            times.append(time.perf_counter() - t0)
+            times.append(max(dt, 1e-9))
     upd = (ext[0] * ext[1] if kind == "fdtd2d" else int(np.prod([e - 2 for e in ext]))) * steps_per
     val = upd * len(times) / sum(times) / 1e9
     line = {"impl": "reference", "metric": METRIC, "value": val, "unit": "GStencil-updates/s",
@@ -235,7 +263,9 @@ def run_reference(args, cfg):
             "config": {"workload": cname, "kind": kind, "extents": list(ext), "T": T},
             "cpu_baseline": {"value": val, "unit": "GStencil-updates/s", "cores": nthreads,
                              "kind": "oracle",
-                             "sample": f"each step = {steps_per} of the workload's {T} time steps on the full grid"},
+                             "sample": f"each step = {steps_per} of the workload's {T} time steps on the full "
+                                       f"grid; the oracle's per-call grid copy-in/out ({overhead * 1e3:.0f} ms, "
+                                       f"measured by 0-step calls) subtracted"},
             "e2e": {"value": val, "unit": "GStencil-updates/s", "h2d_bytes_per_step": 0,
                     "d2h_bytes_per_step": 0}}
     print(json.dumps(line), flush=True)
@@ -272,6 +302,15 @@ def run_gpu(args, cfg):
     one = len(xin) == 1
     stream = torch.cuda.current_stream(dev)
 
+    # L2 hygiene: buffers larger than the 126 MB L2 need nothing; small ones (the 256^2 parity
+    # config) get an L2 flush (a 256 MiB memset) before every timed step, outside its events
+    buf_bytes = sum(x.numel() * x.element_size() for x in xin) * (1 if kind == "fdtd2d" else 2)
+    small = buf_bytes <= 126 * 2**20
+    flush_buf = torch.empty(256 * 2**20, dtype=torch.uint8, device=dev) if small else None
+    nbuf = 3 if kind == "fdtd2d" else 2
+    l2_note = (f"inputs larger than L2 ({nbuf} x {xin[0].numel() * xin[0].element_size() / 2**20:.0f} MiB > 126 MB)"
+               if not small else "L2 flushed (256 MiB memset) before every timed step; per-step events")
+
     def step():
         plan.run(xin[0] if one else xin, xout[0] if one else xout)
 
@@ -282,12 +321,23 @@ def run_gpu(args, cfg):
     start, end = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
     with ClockSampler(local) as clocks:
         torch.cuda.synchronize()
-        start.record(stream)
-        for _ in range(args.steps):
-            step()
-        end.record(stream)
-        torch.cuda.synchronize()
-    ms = start.elapsed_time(end) / args.steps
+        if small:
+            tot = 0.0
+            for _ in range(args.steps):
+                flush_buf.zero_()
+                start.record(stream)
+                step()
+                end.record(stream)
+                torch.cuda.synchronize()
+                tot += start.elapsed_time(end)
+            ms = tot / args.steps
+        else:
+            start.record(stream)
+            for _ in range(args.steps):
+                step()
+            end.record(stream)
+            torch.cuda.synchronize()
+            ms = start.elapsed_time(end) / args.steps
     updates = info["updates"]
     value = updates / (ms * 1e-3) / 1e9
     # ---- per-launch kernel time of the dominant (phase) kernel, live, same stream
@@ -367,7 +417,7 @@ def run_gpu(args, cfg):
         "scaling": "weak", "vs_baseline": None, "dtype": "f32", "data": "synthetic",
         "config": {"workload": cname, "kind": kind, "extents": list(ext), "T": T,
                    "tile": {"h": info["h"], "w0": info["w0"], "w1": info["w"][0]},
-                   "l2": "inputs larger than L2 (2 x 256 MiB ping-pong buffers > 126 MB)"},
+                   "l2": l2_note},
         "roofline": {"bound": "hbm", "achieved": achieved_gbs, "peak": peak, "unit": "GB/s",
                      "frac": achieved_gbs / peak,
                      "traffic": measured_traffic(cfg, {"h": info["h"], "w0": info["w0"]}),

@@ -189,12 +189,14 @@ stencil_status stencil_plan_hexagon(stencil_plan_t plan, int32_t *lo, int32_t *h
 stencil_status stencil_plan_schedule_of(stencil_plan_t plan, int64_t tau, const int64_t *s,
                                         int64_t *sched);
 
-/* Per-launch device timing (used by bench.py for the roofline's kernel time).
- * stencil_plan_profile(plan, max_runs) makes the next max_runs stencil_run calls record a
- * CUDA event pair around every phase-kernel launch on the run's stream (0 disables and
- * frees the events).  stencil_plan_profile_read synchronises on the recorded events and
- * returns the summed kernel time (ms), the number of timed launches and the longest
- * single launch (ms) over the recorded runs, then resets the recorder. */
+/* Device timing of the phase kernels (used by bench.py for the roofline's kernel time).
+ * stencil_plan_profile(plan, max_runs) makes the next max_runs stencil_run calls run eagerly
+ * and record one CUDA event on the run's stream right before its first phase-kernel launch
+ * and one right after its last (the kernel region: every launch of the launch table, back to
+ * back, without the run's boundary copies); 0 disables and frees the events.
+ * stencil_plan_profile_read synchronises on the recorded events and returns the summed
+ * kernel-region time (ms) over the recorded runs, the number of phase-kernel launches they
+ * contain and the longest single run's kernel region (ms), then resets the recorder. */
 stencil_status stencil_plan_profile(stencil_plan_t plan, int max_runs);
 stencil_status stencil_plan_profile_read(stencil_plan_t plan, double *kernel_ms, int64_t *launches,
                                          double *max_launch_ms);

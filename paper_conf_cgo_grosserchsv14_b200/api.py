@@ -164,6 +164,20 @@ class Plan:
             outs = [torch.empty_like(x) for x in ins]
         else:
             outs = [out] if single else list(out)
+            # stencil_run writes whole grids through these pointers: same checks as the inputs
+            if len(outs) != len(ins):
+                raise StencilError(1, f"expected {len(ins)} output field(s)")
+            for o in outs:
+                if not isinstance(o, torch.Tensor) or not o.is_cuda or not o.is_contiguous():
+                    raise StencilError(1, "outputs must be contiguous CUDA tensors")
+                if tuple(o.shape) != self.stencil.extents:
+                    raise StencilError(1, "output shape differs from the descriptor's extents")
+                if _dtype_code(o.dtype) != self.stencil.dtype_code:
+                    raise StencilError(1, "output dtype differs from the descriptor's")
+                if o.device != ins[0].device:
+                    raise StencilError(1, "outputs must live on the inputs' device")
+        if any(x.device != ins[0].device for x in ins):
+            raise StencilError(1, "all input fields must live on one device")
         self._ensure_workspace(ins[0].device)
         n = len(ins)
         in_p = (ctypes.c_void_p * n)(*[x.data_ptr() for x in ins])

@@ -103,6 +103,7 @@ struct Plan {
   std::vector<GraphEntry> graphs;
   int eager_runs = 0;      // runs executed eagerly (the first one sets kernel attributes)
   void* capture_stream = nullptr;
+  int capture_dev = -1;  // device the capture stream was created on
   ~Plan();
 };
 

@@ -1,6 +1,7 @@
 // fast2d_inst.cu -- compiled once per variant id (-DHEXS_VARIANT=<id>); defines
 // hexs::launch_fast2d_v<id>() for the (dtype, class, h, w0, NW) of fast2d_variants.h.
 #include "fast2d_variants.h"
+#include "devcache.h"
 #include "hex2d_impl.cuh"
 
 #ifndef HEXS_VARIANT
@@ -39,20 +40,22 @@ HEXS_CAT(fast2d_kernel_tcut_v, HEXS_VARIANT)(const __grid_constant__ Fast2DArgs 
 }
 
 cudaError_t HEXS_CAT(launch_fast2d_v, HEXS_VARIANT)(const Fast2DArgs& a, int grid, cudaStream_t s) {
-  static bool attr_set = false;
+  static DeviceMemo<int> attr;  // per device: dynamic shared-memory opt-in done
   const int smem = (int)sizeof(KSel::Smem);
-  if (!attr_set) {
-    cudaError_t e = cudaFuncSetAttribute(HEXS_CAT(fast2d_kernel_v, HEXS_VARIANT),
+  int done = 0;
+  cudaError_t e = attr.get(&done, [&](int, int* v) {
+    cudaError_t r = cudaFuncSetAttribute(HEXS_CAT(fast2d_kernel_v, HEXS_VARIANT),
                                          cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
-    if (e == cudaSuccess)
-      e = cudaFuncSetAttribute(HEXS_CAT(fast2d_kernel_unaligned_v, HEXS_VARIANT),
+    if (r == cudaSuccess)
+      r = cudaFuncSetAttribute(HEXS_CAT(fast2d_kernel_unaligned_v, HEXS_VARIANT),
                                cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
-    if (e == cudaSuccess)
-      e = cudaFuncSetAttribute(HEXS_CAT(fast2d_kernel_tcut_v, HEXS_VARIANT),
+    if (r == cudaSuccess)
+      r = cudaFuncSetAttribute(HEXS_CAT(fast2d_kernel_tcut_v, HEXS_VARIANT),
                                cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
-    if (e != cudaSuccess) return e;
-    attr_set = true;
-  }
+    *v = 1;
+    return r;
+  });
+  if (e != cudaSuccess) return e;
   const bool aligned = ((a.N1 * (int64_t)sizeof(KSel::Elem)) % 16) == 0;
   if (a.a_lo > 0 || a.a_hi < KSel::L - 1)
     HEXS_CAT(fast2d_kernel_tcut_v, HEXS_VARIANT)<<<grid, KSel::NT, smem, s>>>(a);

@@ -26,6 +26,7 @@
 #include <cstdint>
 
 #include "../stencil_ops.cuh"
+#include "devcache.h"
 #include "launch.h"
 
 namespace hexs {
@@ -210,13 +211,16 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
 
 template <typename T>
 cudaError_t launch_t(const FdtdArgs& a, int grid, cudaStream_t s) {
-  static size_t attr = 0;
+  // per device: opt in once to the largest ring any plan can ask for (fdtd_variant caps it)
+  static DeviceMemo<int> attr;
   const size_t smem = smem_bytes<T>(a.W);
-  if (smem > attr) {
-    cudaError_t e = cudaFuncSetAttribute(fdtd_kernel<T>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-    if (e != cudaSuccess) return e;
-    attr = smem;
-  }
+  if (smem > 200 * 1024) return cudaErrorInvalidValue;
+  int done = 0;
+  cudaError_t e = attr.get(&done, [](int, int* v) {
+    *v = 1;
+    return cudaFuncSetAttribute(fdtd_kernel<T>, cudaFuncAttributeMaxDynamicSharedMemorySize, 200 * 1024);
+  });
+  if (e != cudaSuccess) return e;
   fdtd_kernel<T><<<grid, NT, smem, s>>>(a);
   return cudaGetLastError();
 }

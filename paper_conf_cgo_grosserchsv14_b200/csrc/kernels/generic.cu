@@ -9,6 +9,7 @@
 // configuration (a), PAPER.md:989 -- and serves as the reference executor for classes
 // without a specialised kernel and as the ablation baseline.
 #include "../stencil_ops.cuh"
+#include "devcache.h"
 #include "launch.h"
 
 namespace hexs {
@@ -223,14 +224,17 @@ __global__ void __launch_bounds__(256) naive_fdtd_kernel(T* __restrict__ ex, T* 
 
 template <typename T, int K>
 int wf_grid_t() {
-  static int grid = 0;
-  if (grid == 0) {
-    int dev = 0, sms = 0, per_sm = 0;
-    cudaGetDevice(&dev);
-    cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
-    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, generic_wf_kernel<T, K>, 256, 0);
-    grid = sms * (per_sm > 0 ? per_sm : 1);
-  }
+  static DeviceMemo<int> memo;  // persistent grid (all CTAs co-resident), per device
+  int grid = 0;
+  if (memo.get(&grid, [](int dev, int* g) {
+        int sms = 0, per_sm = 0;
+        cudaError_t e = cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
+        if (e == cudaSuccess)
+          e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, generic_wf_kernel<T, K>, 256, 0);
+        *g = sms * (per_sm > 0 ? per_sm : 1);
+        return e;
+      }) != cudaSuccess)
+    return 1;
   return grid;
 }
 

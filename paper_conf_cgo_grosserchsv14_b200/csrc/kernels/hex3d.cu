@@ -41,6 +41,7 @@
 
 #include "../stencil_ops.cuh"
 #include "fast3d_variants.h"
+#include "devcache.h"
 #include "launch.h"
 #include "tma.cuh"
 
@@ -684,18 +685,20 @@ template <typename T, int KIND, int H, int W0, int NY, int MINB, int ZS>
 cudaError_t launch_t(const Fast3DArgs& a, cudaStream_t s) {
   using LY = Lay<T, Hex<H, W0>::Q, NY>;
   constexpr int NT = ZS * NY * NQ + 32;  // compute threads + the producer warp
-  static int grid = 0;
+  static DeviceMemo<int> memo;  // per device: smem opt-in + persistent grid size
   constexpr size_t smem = LY::SMEM;
   auto kern = fast3d_kernel<T, KIND, H, W0, NY, MINB, ZS>;
-  if (grid == 0) {
+  int grid = 0;
+  cudaError_t e0 = memo.get(&grid, [&](int dev, int* gsz) {
     cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
     if (e != cudaSuccess) return e;
-    int dev = 0, sms = 0, per_sm = 0;
-    cudaGetDevice(&dev);
-    cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
-    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, NT, smem);
-    grid = sms * (per_sm > 0 ? per_sm : 1);
-  }
+    int sms = 0, per_sm = 0;
+    e = cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
+    if (e == cudaSuccess) e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, NT, smem);
+    *gsz = sms * (per_sm > 0 ? per_sm : 1);
+    return e;
+  });
+  if (e0 != cudaSuccess) return e0;
   if (a.Q != Hex<H, W0>::Q || a.L != Hex<H, W0>::L) return cudaErrorInvalidValue;
   Maps m;
   const uint32_t Q = (uint32_t)a.Q, ny = (uint32_t)NY;

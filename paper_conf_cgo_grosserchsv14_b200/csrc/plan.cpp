@@ -242,8 +242,10 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
       if (p->variant >= 0 && p->hd == 0 && (d.ext[1] * (int64_t)d.elem()) % 16 == 0) ex = EXEC_FDTD;
     } else if (d.dims == 2) {
       p->variant = fast2d_variant(d.kind, dtype, h, w0, t.w[0]);
+      // the kernel's column arithmetic is 32-bit (chunk origins, row bounds): rows of 2^30
+      // columns or more take the generic executor
       if (p->variant >= 0 && p->hd == 0 && p->dcls[0] == 1 && p->d0.n == 1 && p->d0.d == 1 &&
-          p->d1.n == 1 && p->d1.d == 1)
+          p->d1.n == 1 && p->d1.d == 1 && d.ext[1] < (int64_t(1) << 30) && d.ext[0] < (int64_t(1) << 30))
         ex = EXEC_FAST2D;
     } else {
       p->variant = fast3d_variant(d.kind, dtype, h, w0, t.w[0]);

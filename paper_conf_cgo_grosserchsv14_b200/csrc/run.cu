@@ -67,19 +67,21 @@ static int64_t launches_per_run(const Plan& p) {
 
 stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* stream_) {
   const Desc& d = p.desc;
-  // optional per-launch event pairs (stencil_plan_profile)
+  // optional kernel-region events (stencil_plan_profile): one event before the first phase
+  // kernel of the run and one after the last, on the run's stream
   cudaEvent_t* ev = nullptr;
   if (p.prof_runs > 0 && p.prof_used < p.prof_runs) {
-    ev = reinterpret_cast<cudaEvent_t*>(p.prof_events.data()) + (size_t)p.prof_used * 2 * launches_per_run(p);
+    ev = reinterpret_cast<cudaEvent_t*>(p.prof_events.data()) + (size_t)p.prof_used * 2;
     p.prof_used++;
   }
+  const int64_t n_launch = launches_per_run(p);
   int64_t li = 0;
   auto ev_begin = [&](cudaStream_t st) {
-    if (ev) cudaEventRecord(ev[2 * li], st);
+    if (ev && li == 0) cudaEventRecord(ev[0], st);
   };
   auto ev_end = [&](cudaStream_t st) {
-    if (ev) cudaEventRecord(ev[2 * li + 1], st);
     ++li;
+    if (ev && li == n_launch) cudaEventRecord(ev[1], st);
   };
   cudaStream_t s = static_cast<cudaStream_t>(stream_);
   const size_t bytes = (size_t)d.points() * d.elem();
@@ -252,10 +254,18 @@ extern "C" stencil_status stencil_run(stencil_plan_t plan, const void* const* in
       return STENCIL_OK;
     }
   if (p->eager_runs++ == 0 || p->graphs.size() >= 8) return run_plan(*p, in, out, stream);
+  // the private capture stream lives on the device the plan currently runs on
+  int dev = -1;
+  HEXS_CUDA(cudaGetDevice(&dev), "stencil_run: no CUDA device");
+  if (p->capture_stream && p->capture_dev != dev) {
+    cudaStreamDestroy(static_cast<cudaStream_t>(p->capture_stream));
+    p->capture_stream = nullptr;
+  }
   if (!p->capture_stream) {
     cudaStream_t cs = nullptr;
     HEXS_CUDA(cudaStreamCreateWithFlags(&cs, cudaStreamNonBlocking), "stencil_run: capture stream");
     p->capture_stream = cs;
+    p->capture_dev = dev;
   }
   cudaStream_t cs = static_cast<cudaStream_t>(p->capture_stream);
   HEXS_CUDA(cudaStreamBeginCapture(cs, cudaStreamCaptureModeThreadLocal), "stencil_run: begin capture");
@@ -263,8 +273,12 @@ extern "C" stencil_status stencil_run(stencil_plan_t plan, const void* const* in
   cudaGraph_t graph = nullptr;
   const cudaError_t ec = cudaStreamEndCapture(cs, &graph);
   if (st != STENCIL_OK) {
+    // a launch failed while capturing: drop the partial graph and run eagerly on the
+    // caller's stream (a genuine error surfaces again there)
     if (graph) cudaGraphDestroy(graph);
-    return st;
+    cudaGetLastError();
+    clear_error();
+    return run_plan(*p, in, out, stream);
   }
   if (ec != cudaSuccess || !graph) {
     cudaGetLastError();
@@ -292,7 +306,7 @@ extern "C" stencil_status stencil_plan_profile(stencil_plan_t plan, int max_runs
   p->prof_runs = 0;
   p->prof_used = 0;
   if (max_runs == 0) return STENCIL_OK;
-  const size_t n = (size_t)max_runs * 2 * launches_per_run(*p);
+  const size_t n = (size_t)max_runs * 2;
   p->prof_events.assign(n, nullptr);
   for (size_t i = 0; i < n; ++i) {
     cudaEvent_t e;
@@ -310,10 +324,10 @@ extern "C" stencil_status stencil_plan_profile_read(stencil_plan_t plan, double*
   Plan* p = reinterpret_cast<Plan*>(plan);
   if (!p || p->magic != kPlanMagic || !kernel_ms || !launches || !max_launch_ms)
     return fail(STENCIL_E_INVALID, "stencil_plan_profile_read: bad arguments");
-  const int64_t n = (int64_t)p->prof_used * launches_per_run(*p);
+  const int64_t runs = p->prof_used, per = launches_per_run(*p);
   double total = 0, mx = 0;
   cudaEvent_t* ev = reinterpret_cast<cudaEvent_t*>(p->prof_events.data());
-  for (int64_t i = 0; i < n; ++i) {
+  for (int64_t i = 0; i < runs && per > 0; ++i) {
     HEXS_CUDA(cudaEventSynchronize(ev[2 * i + 1]), "stencil_plan_profile_read: sync");
     float ms = 0;
     HEXS_CUDA(cudaEventElapsedTime(&ms, ev[2 * i], ev[2 * i + 1]), "stencil_plan_profile_read: elapsed");
@@ -321,7 +335,7 @@ extern "C" stencil_status stencil_plan_profile_read(stencil_plan_t plan, double*
     if (ms > mx) mx = ms;
   }
   *kernel_ms = total;
-  *launches = n;
+  *launches = per > 0 ? runs * per : 0;
   *max_launch_ms = mx;
   p->prof_used = 0;
   return STENCIL_OK;

@@ -220,7 +220,10 @@ def bench_main(args, cfg, configs, metric, helpers=None):
         k = i % 2
         with torch.cuda.stream(h2d):
             if i >= 2:
+                # the slab buffer is both input and output: its previous step's compute AND
+                # the download of that step's result must be done before it is overwritten
                 h2d.wait_event(ev_done[k])
+                h2d.wait_event(ev_out[k])
             locs[k].copy_(host_in, non_blocking=True)
             ev_in[k].record(h2d)
         stream.wait_event(ev_in[k])
@@ -239,6 +242,11 @@ def bench_main(args, cfg, configs, metric, helpers=None):
     e2e_ms = torch.tensor([f0.elapsed_time(f1) / args.steps], device="cuda")
     dist.all_reduce(e2e_ms, op=dist.ReduceOp.MAX)
     e2e_ms = float(e2e_ms.item())
+    # the pipelined result equals a device-resident run's owned planes
+    ref = local0.clone()
+    runner.run(ref)
+    torch.cuda.synchronize()
+    assert torch.equal(host_out[(args.steps - 1) % 2], ref[lo:hi].cpu()), "pipelined e2e result differs"
     host_out = host_out[0]
 
     # phase-kernel roofline of the main block plan (algorithmic bytes / measured launch time)
