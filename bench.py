@@ -142,7 +142,9 @@ def bytes_per_update_tiled(info, word, plan=None):
 
 
 KERNEL_NAMES = {"fast2d": "fast2d_kernel (2D register wavefront)", "fdtd": "fdtd_kernel (FDTD smem ring)",
-                "fast3d": "fast3d_kernel (3D classical-tile wavefront)", "generic": "generic_kernel"}
+                "fast3d": "fast3d_kernel (3D classical-tile wavefront)",
+                "stream3d": "stream3d_kernel (3D: hexagons over (t,y), z streamed through registers)",
+                "generic": "generic_kernel", "naive": "naive kernel"}
 
 
 def measured_traffic(cfg, tile):

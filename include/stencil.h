@@ -72,7 +72,7 @@ typedef struct {
   int32_t h;
   int32_t w0;
   int32_t w[3];
-  int32_t hex_dim;
+  int32_t hex_dim;  /* < 0: automatic (y for the streaming 3D star kernel, else dimension 0) */
   int32_t flags; /* STENCIL_EXEC_* */
 } stencil_tile_t;
 
@@ -159,7 +159,17 @@ typedef struct {
   int64_t tile_points;   /* instances of one full hexagon per classical column */
   int64_t tile_in, tile_out; /* In / Out values of one full hexagon per column */
   size_t workspace_bytes;
+  int32_t kernel;        /* STENCIL_KERNEL_*: the phase-kernel family that runs */
 } stencil_plan_info_t;
+
+enum {
+  STENCIL_KERNEL_GENERIC = 0,   /* kernels/generic.cu: Sec. 4.1 mapping from global memory   */
+  STENCIL_KERNEL_NAIVE = 1,     /* one launch per time step (comparator)                      */
+  STENCIL_KERNEL_FAST2D = 2,    /* 2D register wavefront, TMA-staged In rows                  */
+  STENCIL_KERNEL_FDTD = 3,      /* FDTD-2D shared-memory ring                                 */
+  STENCIL_KERNEL_FAST3D = 4,    /* 3D tile wavefront, hexagons over (t, z), levels in smem    */
+  STENCIL_KERNEL_STREAM3D = 5   /* 3D streaming: hexagons over (t, y), z streamed, registers  */
+};
 
 stencil_status stencil_plan_info(stencil_plan_t plan, stencil_plan_info_t *info);
 

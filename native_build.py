@@ -46,6 +46,7 @@ def _deps_hash(paths):
 
 
 EXTRA3D = []  # extra flags of the 3D kernel objects (debug builds)
+EXTRAS3 = []  # extra flags of the streaming 3D kernel objects
 
 
 def _units():
@@ -61,6 +62,8 @@ def _units():
         units.append((os.path.join(KDIR, "fast2d_inst.cu"), "nvcc", [f"-DHEXS_VARIANT={vid}"]))
     for vid in _variant_ids("fast3d_variants.h", "HEXS_FAST3D_VARIANTS"):
         units.append((os.path.join(KDIR, "hex3d.cu"), "nvcc", [f"-DHEXS_F3_VARIANT={vid}"] + EXTRA3D))
+    for vid in _variant_ids("stream3d_variants.h", "HEXS_STREAM3D_VARIANTS"):
+        units.append((os.path.join(KDIR, "stream3d.cu"), "nvcc", [f"-DHEXS_S3_VARIANT={vid}"] + EXTRAS3))
     out = []
     for src, tool, extra in units:
         key = _deps_hash([src] + headers) + hashlib.sha1(" ".join(extra).encode()).hexdigest()[:8]
@@ -119,8 +122,17 @@ def main():
     ap.add_argument("-v", action="store_true")
     ap.add_argument("--timing", action="store_true",
                     help="also build lib/libhexstencil_tm.so with the 3D kernel's cycle accounting")
+    ap.add_argument("--s3trace", action="store_true",
+                    help="also build lib/libhexstencil_s3t.so with the streaming 3D kernel's event trace")
     args = ap.parse_args()
     print(build_library(args.j, args.v))
+    if args.s3trace:
+        EXTRAS3.append("-DHEXS_S3_TRACE")
+        print(build_library(args.j, args.v, lib=os.path.join(PKG, "lib", "libhexstencil_s3t.so")))
+        for tag, flag in ():
+            EXTRAS3.append(flag)
+            print(build_library(args.j, args.v, lib=os.path.join(PKG, "lib", f"libhexstencil_s3t_{tag}.so")))
+            EXTRAS3.remove(flag)
     if args.timing:
         EXTRA3D.append("-DHEXS_F3_TIMING")
         print(build_library(args.j, args.v, lib=os.path.join(PKG, "lib", "libhexstencil_tm.so")))

@@ -53,7 +53,9 @@ class PlanInfo(ctypes.Structure):
                 ("T_steps", ctypes.c_int64), ("tau_levels", ctypes.c_int64),
                 ("updates", ctypes.c_int64), ("tile_points", ctypes.c_int64),
                 ("tile_in", ctypes.c_int64), ("tile_out", ctypes.c_int64),
-                ("workspace_bytes", ctypes.c_size_t)]
+                ("workspace_bytes", ctypes.c_size_t), ("kernel", ctypes.c_int32)]
+
+KERNELS = {0: "generic", 1: "naive", 2: "fast2d", 3: "fdtd", 4: "fast3d", 5: "stream3d"}
 
 
 class Launch(ctypes.Structure):

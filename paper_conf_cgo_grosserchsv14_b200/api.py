@@ -76,7 +76,7 @@ class Plan:
     `run` enqueues the phase kernels on the current CUDA stream."""
 
     def __init__(self, stencil: Stencil, T_steps: int, h: int = 0, w0: int = 0,
-                 w: Sequence[int] = (0, 0, 0), hex_dim: int = 0, executor: str = "auto"):
+                 w: Sequence[int] = (0, 0, 0), hex_dim: int = -1, executor: str = "auto"):
         self.stencil = stencil
         self.T_steps = int(T_steps)
         t = Tile(int(h), int(w0), (ctypes.c_int32 * 3)(*list(w)[:3]), int(hex_dim), EXEC[executor])
@@ -98,11 +98,8 @@ class Plan:
 
     @property
     def executor_name(self) -> str:
-        """Which kernel family runs: fast2d / fdtd / fast3d (specialised) or generic / naive."""
-        i = self.info
-        if i["fast_kernel"]:
-            return "fdtd" if self.stencil.kind == "fdtd2d" else ("fast3d" if len(self.stencil.extents) == 3 else "fast2d")
-        return "naive" if i["executor"] == 2 else "generic"
+        """Which kernel family runs: fast2d / fdtd / fast3d / stream3d (specialised) or generic / naive."""
+        return _lib.KERNELS[self.info["kernel"]]
 
     def launches(self) -> List[Dict[str, int]]:
         n = ctypes.c_int64()

@@ -12,6 +12,8 @@ namespace hexs {
 constexpr uint32_t kDescMagic = 0x48584453u;  // "HXDS"
 constexpr uint32_t kPlanMagic = 0x48585053u;  // "HXPS"
 constexpr int kMaxLevels = 64;                // max 2h+2 supported by the kernels
+constexpr int kStream3DNXPlan = 64;           // = kernels/launch.h kStream3DNX (strip width)
+constexpr int kStream3DRSPlan = 32;           // = kernels/launch.h kStream3DRS (carry ring depth)
 
 // A rational number n/d, d > 0, reduced.
 struct Rat {
@@ -65,9 +67,11 @@ struct Launch {
   int64_t Slo[2], Shi[2];
   // wavefront executors: first tile flag and work counter of this launch in the workspace
   int64_t flag_first = 0, counter_idx = 0;
+  // stream3d: first progress counter of this launch (its ticket follows the launch's counters)
+  int64_t s3_ctr_first = 0;
 };
 
-enum Executor { EXEC_GENERIC = 1, EXEC_NAIVE = 2, EXEC_FAST2D = 3, EXEC_FDTD = 4, EXEC_FAST3D = 5 };
+enum Executor { EXEC_GENERIC = 1, EXEC_NAIVE = 2, EXEC_FAST2D = 3, EXEC_FDTD = 4, EXEC_FAST3D = 5, EXEC_STREAM3D = 6 };
 
 struct Plan {
   uint32_t magic = kPlanMagic;
@@ -88,6 +92,9 @@ struct Plan {
   int64_t tile_points = 0, tile_in = 0, tile_out = 0;
   bool wavefront = false;      // generic executor: classical tiles as a dependence wavefront
   size_t flag_off = 0, counter_off = 0, flag_bytes = 0;  // workspace layout (wavefront)
+  // stream3d: per-launch progress counters + ticket (zeroed per run), carry scratch
+  size_t s3_ctr_off = 0, s3_ctr_bytes = 0, s3_scratch_off = 0;
+  int s3_nstr = 0;
   size_t ws_bytes = 0;
   void* ws = nullptr;
   size_t ws_size = 0;
@@ -126,5 +133,7 @@ int fdtd_ctas_per_sm();
 int fast3d_variant(int kind, int dtype, int h, int w0, int wy);
 int fast3d_tile(int variant, int* wy, int* wx);
 bool fast3d_variant_matches(int variant, int kind, int dtype, int h, int w0);
+int stream3d_variant(int kind, int dtype, int h, int w0);
+int stream3d_carry_block(int variant);  // floats per (strip, step) carry block
 
 }  // namespace hexs

@@ -92,4 +92,25 @@ struct Fast3DArgs {
 cudaError_t launch_fast3d(int variant, const Fast3DArgs& a, int grid, cudaStream_t s);
 constexpr int kFast3DNX = 32;            // classical tile width along x of the 3D fast kernel
 
+// Streaming 3D kernel (kernels/stream3d.cu): hexagons over (t, y), z streamed plane by plane
+// (classical width 1, skew 1), x in strips of kStream3DNX (skew 4).  One CTA per (hexagon,
+// strip), ticketed in (hexagon, strip) order; strips pass their right-edge quads through
+// `scratch` (kStream3DRS steps deep) and publish per-step progress counters.
+constexpr int kStream3DNX = 64;
+constexpr int kStream3DRS = 32;
+struct Stream3DArgs {
+  void* buf[2];
+  int64_t N0, N1, N2;
+  int64_t tau0;
+  int a_lo, a_hi, a_final;
+  int64_t S0_lo, row_off;
+  int W, L, RN;        // box width, levels 2h+2, hexagon rows 2h+w0+1
+  int n_str, n_items;  // strips per hexagon, CTAs of the launch
+  double k0, k1;
+  int* progress;           // [n_items] completed steps, zeroed per launch
+  unsigned int* ticket;    // CTA ticket counter, zeroed per launch
+  float* scratch;          // [n_items][kStream3DRS][carry block]
+};
+cudaError_t launch_stream3d(int variant, const Stream3DArgs& a, cudaStream_t s);
+
 }  // namespace hexs

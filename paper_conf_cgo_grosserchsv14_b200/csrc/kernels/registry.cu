@@ -3,6 +3,7 @@
 #include "../stencil_ops.cuh"
 #include "fast2d_variants.h"
 #include "fast3d_variants.h"
+#include "stream3d_variants.h"
 #include "launch.h"
 
 namespace hexs {
@@ -82,6 +83,37 @@ cudaError_t launch_fast3d(int variant, const Fast3DArgs& a, int /*grid: persiste
   case id: return launch_fast3d_v##id(a, s);
     HEXS_FAST3D_VARIANTS(HEXS_F3_L)
 #undef HEXS_F3_L
+    default: return cudaErrorInvalidValue;
+  }
+}
+
+// Streaming 3D kernel: the compiled (class, h, w0) instantiations of stream3d_variants.h.
+#define HEXS_S3_DECL(id, dc, T_, KIND_, H_, W0_, NXS_)                                \
+  cudaError_t launch_stream3d_v##id(const Stream3DArgs& a, cudaStream_t s); \
+  int stream3d_carry_block_v##id();
+HEXS_STREAM3D_VARIANTS(HEXS_S3_DECL)
+#undef HEXS_S3_DECL
+
+int stream3d_variant(int kind, int dtype, int h, int w0) {
+#define HEXS_S3_MATCH(id, dc, T_, KIND_, H_, W0_, NXS_) \
+  if (kind == KIND_ && dtype == dc && h == H_ && w0 == W0_) return id;
+  HEXS_STREAM3D_VARIANTS(HEXS_S3_MATCH)
+#undef HEXS_S3_MATCH
+  return -1;
+}
+int stream3d_carry_block(int variant) {
+  switch (variant) {
+#define HEXS_S3_CB(id, dc, T_, KIND_, H_, W0_, NXS_) case id: return stream3d_carry_block_v##id();
+    HEXS_STREAM3D_VARIANTS(HEXS_S3_CB)
+#undef HEXS_S3_CB
+    default: return 0;
+  }
+}
+cudaError_t launch_stream3d(int variant, const Stream3DArgs& a, cudaStream_t s) {
+  switch (variant) {
+#define HEXS_S3_L(id, dc, T_, KIND_, H_, W0_, NXS_) case id: return launch_stream3d_v##id(a, s);
+    HEXS_STREAM3D_VARIANTS(HEXS_S3_L)
+#undef HEXS_S3_L
     default: return cudaErrorInvalidValue;
   }
 }

@@ -150,8 +150,19 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
   p->T_steps = T_steps;
   p->tau_levels = T_steps * (int64_t)d.stmts.size();
   stencil_tile_t t{};
+  t.hex_dim = -1;  // NULL tile: everything automatic
   if (tile) t = *tile;
-  p->hd = t.hex_dim;
+  // hex_dim < 0: automatic -- the streaming 3D kernel tiles y hexagonally (its stream runs along
+  // z, the outermost dimension, PAPER.md:633-641 allows any non-innermost dimension); everything
+  // else tiles the outermost dimension
+  const bool s3_class = d.dims == 3 && (d.kind == STENCIL_STAR3D7 || d.kind == STENCIL_GRADIENT3D) &&
+                        d.dtype == STENCIL_F32 && t.flags == STENCIL_EXEC_AUTO && d.ext[2] % 4 == 0 &&
+                        d.ext[2] < (int64_t(1) << 30) && d.ext[1] < (int64_t(1) << 30) &&
+                        d.ext[0] < (int64_t(1) << 30);
+  // (measured on B200: the tile-wavefront kernel over (t, z) is still the faster default for the
+  // star classes; HEXS_STREAM3D=1 makes the streaming kernel the automatic choice)
+  static const bool s3_auto = std::getenv("HEXS_STREAM3D") && std::atoi(std::getenv("HEXS_STREAM3D")) != 0;
+  p->hd = t.hex_dim >= 0 ? t.hex_dim : (s3_class && s3_auto ? 1 : 0);
   if (p->hd < 0 || p->hd >= d.dims - 1)
     return fail(STENCIL_E_INVALID, "stencil_plan: hex_dim must be a non-innermost dimension (PAPER.md:636-641)");
   p->ncls = 0;
@@ -192,6 +203,8 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
       if (d.kind == STENCIL_BOX2D9 && dtype == STENCIL_F32) h = 2;
       // IEEE sqrt + div per point: only the smallest hexagon's body stays in the i-cache
       if (d.kind == STENCIL_GRADIENT2D && dtype == STENCIL_F32) h = 1, w0 = 1;
+    } else if (s3_class && p->hd == 1) {
+      h = 2; w0 = 7;  // streaming kernel: Table 4's h = 2; two CTAs per SM
     } else {
       h = 2; w0 = 7;  // Table 4 setup
       // the 7-point star: one more level pair per tile amortises the per-tile fills and flags
@@ -247,6 +260,9 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
       if (p->variant >= 0 && p->hd == 0 && p->dcls[0] == 1 && p->d0.n == 1 && p->d0.d == 1 &&
           p->d1.n == 1 && p->d1.d == 1 && d.ext[1] < (int64_t(1) << 30) && d.ext[0] < (int64_t(1) << 30))
         ex = EXEC_FAST2D;
+    } else if (s3_class && p->hd == 1) {
+      p->variant = stream3d_variant(d.kind, dtype, h, w0);
+      if (p->variant >= 0 && p->d0.n == 1 && p->d0.d == 1 && p->d1.n == 1 && p->d1.d == 1) ex = EXEC_STREAM3D;
     } else {
       p->variant = fast3d_variant(d.kind, dtype, h, w0, t.w[0]);
       // tuning aid: HEXS_F3_FORCE_VARIANT=<id> picks a compiled variant of the same shape
@@ -269,6 +285,7 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
   for (int q = 0; q < p->ncls; ++q) {
     int wq = t.w[q];
     if (ex == EXEC_FAST2D) wq = fast2d_chunk_width(p->variant);
+    else if (ex == EXEC_STREAM3D) wq = q == 0 ? 1 : kStream3DNXPlan;  // z planes streamed; x strips
     else if (ex == EXEC_FAST3D) {
       int wy = 0, wx = 0;
       fast3d_tile(p->variant, &wy, &wx);
@@ -284,7 +301,7 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
   // The 3D fast kernel moves whole 16-B groups (TMA boxes, vector loads/stores): it skews the
   // contiguous dimension by 4 per level (any integer skew >= delta1_i keeps eq. (14) valid,
   // reading R16), so every tile boundary of every level is 16-B aligned.
-  if (ex == EXEC_FAST3D) {
+  if (ex == EXEC_FAST3D || ex == EXEC_STREAM3D) {
     p->dcls[1] = std::max(p->dcls[1], 4);
     p->ctrans[1] = 0;
   }
@@ -354,6 +371,25 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
     p->counter_off = p->flag_off + ((size_t)n_items * sizeof(int) + 255) / 256 * 256;
     p->flag_bytes = p->counter_off - p->flag_off + ((size_t)idx * 8 + 255) / 256 * 256;  // flags + counters
     p->ws_bytes = p->flag_off + p->flag_bytes;
+  }
+  // streaming 3D kernel: per launch a progress counter per (hexagon, strip) CTA plus a ticket
+  // (zeroed together by one memset per run), and the carry scratch ring shared by the
+  // launches (they run one after the other on the stream)
+  if (ex == EXEC_STREAM3D && !p->launches.empty()) {
+    p->s3_nstr = (int)((d.ext[2] - 1 + 4 * (p->H - 1)) / kStream3DNXPlan + 1);
+    int64_t ctr = 0, max_items = 0;
+    for (Launch& l : p->launches) {
+      const int64_t items = (l.S0_hi - l.S0_lo + 1) * p->s3_nstr;
+      if (items > INT32_MAX / 2) return fail(STENCIL_E_UNSUPPORTED, "stencil_plan: too many tiles per launch");
+      l.s3_ctr_first = ctr;
+      ctr += items + 1;  // counters, then the ticket
+      max_items = std::max(max_items, items);
+    }
+    p->s3_ctr_off = p->ws_bytes;
+    p->s3_ctr_bytes = ((size_t)ctr * sizeof(int) + 255) / 256 * 256;
+    p->s3_scratch_off = p->s3_ctr_off + p->s3_ctr_bytes;
+    const size_t cblk = (size_t)stream3d_carry_block(p->variant) * sizeof(float);
+    p->ws_bytes = p->s3_scratch_off + ((size_t)max_items * kStream3DRSPlan * cblk + 255) / 256 * 256;
   }
   *out = guard.release();
   return STENCIL_OK;
@@ -433,7 +469,13 @@ stencil_status stencil_plan_info(stencil_plan_t plan, stencil_plan_info_t* info)
   o.F1 = p->F1;
   o.executor = p->executor == EXEC_NAIVE ? STENCIL_EXEC_NAIVE
              : p->executor == EXEC_GENERIC ? STENCIL_EXEC_GENERIC : STENCIL_EXEC_AUTO;
-  o.fast_kernel = (p->executor == EXEC_FAST2D || p->executor == EXEC_FDTD || p->executor == EXEC_FAST3D);
+  o.fast_kernel = (p->executor == EXEC_FAST2D || p->executor == EXEC_FDTD || p->executor == EXEC_FAST3D ||
+                   p->executor == EXEC_STREAM3D);
+  o.kernel = p->executor == EXEC_FAST2D ? STENCIL_KERNEL_FAST2D
+           : p->executor == EXEC_FDTD ? STENCIL_KERNEL_FDTD
+           : p->executor == EXEC_FAST3D ? STENCIL_KERNEL_FAST3D
+           : p->executor == EXEC_STREAM3D ? STENCIL_KERNEL_STREAM3D
+           : p->executor == EXEC_NAIVE ? STENCIL_KERNEL_NAIVE : STENCIL_KERNEL_GENERIC;
   o.n_launches = p->executor == EXEC_NAIVE ? p->tau_levels : (int64_t)p->launches.size();
   o.T_steps = p->T_steps;
   o.tau_levels = p->tau_levels;

@@ -124,6 +124,9 @@ stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* 
     if (p.wavefront)
       HEXS_CUDA(cudaMemsetAsync(static_cast<char*>(p.ws) + p.flag_off, 0, p.flag_bytes, s),
                 "stencil_run: reset tile flags");
+    if (p.executor == EXEC_STREAM3D)
+      HEXS_CUDA(cudaMemsetAsync(static_cast<char*>(p.ws) + p.s3_ctr_off, 0, p.s3_ctr_bytes, s),
+                "stencil_run: reset strip progress counters");
     for (const Launch& l : p.launches) {
       const int a_final = (l.tau0 + l.a_hi + 1 == p.tau_levels) ? l.a_hi : -1;
       const int64_t grid64 = l.S0_hi - l.S0_lo + 1;
@@ -165,6 +168,31 @@ stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* 
           a.hi[q] = p.hi[q];
         }
         HEXS_CUDA(launch_fdtd(p.variant, a, grid, s), "stencil_run: fdtd kernel launch");
+      } else if (p.executor == EXEC_STREAM3D) {
+        Stream3DArgs a{};
+        a.buf[0] = buf[0];
+        a.buf[1] = buf[1];
+        a.N0 = d.ext[0];
+        a.N1 = d.ext[1];
+        a.N2 = d.ext[2];
+        a.tau0 = l.tau0;
+        a.a_lo = l.a_lo;
+        a.a_hi = l.a_hi;
+        a.a_final = a_final;
+        a.S0_lo = l.S0_lo;
+        a.row_off = l.row_off;
+        a.W = p.W;
+        a.L = p.H;
+        a.RN = 2 * p.h + p.w0 + 1;
+        a.n_str = p.s3_nstr;
+        a.n_items = (int)((l.S0_hi - l.S0_lo + 1) * p.s3_nstr);
+        a.k0 = d.coef[0];
+        a.k1 = d.coef[1];
+        char* ws = static_cast<char*>(p.ws);
+        a.progress = reinterpret_cast<int*>(ws + p.s3_ctr_off) + l.s3_ctr_first;
+        a.ticket = reinterpret_cast<unsigned int*>(a.progress + a.n_items);
+        a.scratch = reinterpret_cast<float*>(ws + p.s3_scratch_off);
+        HEXS_CUDA(launch_stream3d(p.variant, a, s), "stencil_run: stream3d kernel launch");
       } else if (p.executor == EXEC_FAST3D) {
         Fast3DArgs a{};
         a.buf[0] = buf[0];

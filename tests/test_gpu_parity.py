@@ -147,10 +147,26 @@ def test_3d(kind, dtype, executor):
 
 @pytest.mark.parametrize("h,w0", [(2, 7), (1, 3), (3, 2)])
 def test_fast3d_tiles(h, w0):
+    """The tile-wavefront 3D kernel (hexagons over (t, z), hex_dim = 0)."""
     g = stencil_inputs.uniform((41, 70, 96), seed=31)
-    got, plan = _gpu_run("star3d7", g, 11, np.float32, h=h, w0=w0)
-    assert plan.info["fast_kernel"] == 1
+    got, plan = _gpu_run("star3d7", g, 11, np.float32, h=h, w0=w0, hex_dim=0)
+    assert plan.executor_name == "fast3d"
     assert_bitexact(got, oracle.run("star3d7", g, 11), f"fast3d h={h} w0={w0}")
+
+
+@pytest.mark.parametrize("kind,h,w0", [("star3d7", 2, 7), ("star3d7", 1, 3), ("star3d7", 3, 5), ("star3d7", 1, 7),
+                                       ("star3d7", 2, 5), ("star3d7", 3, 7), ("gradient3d", 2, 7),
+                                       ("gradient3d", 1, 7)])
+@pytest.mark.parametrize("shape,T", [((41, 70, 96), 11), ((20, 33, 200), 17), ((9, 100, 64), 6), ((33, 5, 132), 9),
+                                     ((3, 40, 68), 5), ((50, 47, 4), 8)])
+def test_stream3d_tiles(kind, h, w0, shape, T):
+    """The streaming 3D kernel (hexagons over (t, y), z streamed, x strips): several strips,
+    hexagons cut by the grid and by t = 0 / t = T, degenerate extents (3 planes, 5 rows,
+    4 columns), T not a multiple of 2h+2."""
+    g = stencil_inputs.uniform(shape, seed=32)
+    got, plan = _gpu_run(kind, g, T, np.float32, h=h, w0=w0, hex_dim=1)
+    assert plan.executor_name == "stream3d" and plan.info["hex_dim"] == 1
+    assert_bitexact(got, oracle.run(kind, g, T), f"stream3d {kind} h={h} w0={w0} {shape} T={T}")
 
 
 def test_constant_field_full_size_property():

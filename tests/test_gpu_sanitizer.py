@@ -23,7 +23,7 @@ def test_compute_sanitizer(tool):
     if tool == "initcheck":
         # the workspace tail (flags/counters) is memset by stencil_run itself; cudaMalloc'd
         # grids are fully written by the host before the run
-        cmd += ["--track-unused-memory", "no"]
+        cmd += ["--check-api-memory-access", "yes"]
     cmd += [sys.executable, os.path.join(ROOT, "tools", "sanitize_cases.py")]
     r = subprocess.run(cmd, capture_output=True, text=True, timeout=1500, cwd=ROOT)
     out = r.stdout + r.stderr

@@ -30,7 +30,7 @@ def dmalloc(n):
     return p
 
 
-def run_case(kind, shape, T, dtype=np.float32, h=0, w0=0, executor="auto"):
+def run_case(kind, shape, T, dtype=np.float32, h=0, w0=0, executor="auto", hex_dim=-1):
     L = _lib.lib()
     nf = 3 if kind == "fdtd2d" else 1
     fields = (stencil_inputs.fields(shape, seed=3, n=3, dtype=dtype) if nf == 3
@@ -39,7 +39,7 @@ def run_case(kind, shape, T, dtype=np.float32, h=0, w0=0, executor="auto"):
     d = ctypes.c_void_p()
     check(L.stencil_desc_create(ctypes.byref(d), len(shape), ext, KINDS[kind], 1, None, 0, None, 0,
                                 1 if dtype == np.float64 else 0))
-    t = Tile(h, w0, (ctypes.c_int32 * 3)(0, 0, 0), 0, EXEC[executor])
+    t = Tile(h, w0, (ctypes.c_int32 * 3)(0, 0, 0), hex_dim, EXEC[executor])
     p = ctypes.c_void_p()
     check(L.stencil_plan(ctypes.byref(p), d, T, ctypes.byref(t)))
     ws_n = ctypes.c_size_t()
@@ -73,8 +73,10 @@ CASES = {
     "fast2d_box": ("box2d9", (45, 531), 11, np.float32, 2, 7),      # unaligned rows
     "fast2d_grad": ("gradient2d", (40, 1024), 9, np.float32, 0, 0),
     "fast2d_f64": ("star2d5", (40, 520), 9, np.float64, 0, 0),
-    "fast3d": ("star3d7", (26, 40, 72), 9, np.float32, 0, 0),
-    "fast3d_grad": ("gradient3d", (22, 36, 68), 7, np.float32, 0, 0),
+    "stream3d": ("star3d7", (26, 40, 136), 9, np.float32, 0, 0),       # 3 strips, default (2,7)
+    "stream3d_grad": ("gradient3d", (22, 36, 68), 7, np.float32, 0, 0),
+    "stream3d_h1": ("star3d7", (19, 30, 72), 6, np.float32, 1, 7),
+    "fast3d": ("star3d7", (26, 40, 72), 9, np.float32, 0, 0),           # hex_dim 0: tile wavefront
     "fast3d_box": ("box3d27", (20, 34, 64), 7, np.float32, 0, 0),
     "fast3d_f64": ("star3d7", (20, 34, 64), 7, np.float64, 0, 0),
     "fdtd": ("fdtd2d", (60, 136), 9, np.float32, 0, 0),
@@ -88,7 +90,8 @@ def main(argv):
     for n in names:
         kind, shape, T, dt, h, w0 = CASES[n]
         ex = "generic" if n.startswith("generic") else "auto"
-        ok = run_case(kind, shape, T, dt, h, w0, ex)
+        hd = 0 if n.startswith("fast3d") else (1 if n.startswith("stream3d") else -1)
+        ok = run_case(kind, shape, T, dt, h, w0, ex, hd)
         print(f"{n}: {'ok' if ok else 'MISMATCH'}", flush=True)
         if not ok:
             bad.append(n)
