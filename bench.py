@@ -35,7 +35,15 @@ CONFIGS = {
     # the rest of the paper's Table 3 workload set, same grid sizes
     "heat3d27": ("box3d27", (512, 512, 512), 128, "heat-3D 27-point fp32 (the paper's heat 3D), 512^3, T=128"),
     "gradient2d": ("gradient2d", (8192, 8192), 512, "gradient-2D fp32, 8192x8192, T=512"),
+    # configs[4]: the slab-partitioned 3D grids (multi-GPU slab mode); strong
+    # scaling of 1024^3 and weak scaling of 256*P x 1024^2 (2048 x 1024^2 at P = 8)
+    "heat3d1024": ("star3d7", (1024, 1024, 1024), 256,
+                   "heat-3D 7-point fp32, 1024^3, T=256, slab-partitioned", "strong"),
+    "heat3d_weak": ("star3d7", (256, 1024, 1024), 256,
+                    "heat-3D 7-point fp32, 256*P x 1024^2 (2048x1024^2 at P=8), T=256, slab-partitioned", "weak"),
 }
+# configs that always run through the distributed plan (stencil_plan_dist), also at N = 1
+DIST_CONFIGS = {"heat3d1024", "heat3d_weak"}
 METRIC = "GStencil-updates/s (fp32) at 1/2/4/8 B200 and % of time-tiled HBM roofline"
 
 
@@ -229,7 +237,7 @@ def run_reference(args, cfg):
     (about a second of work).  oracle.run copies the grid in and out on every call; that fixed
     per-call cost is measured with 0-step calls and subtracted, so the number is the oracle's
     time-stepping rate (what cpu_baseline reports), not its argument marshalling."""
-    kind, ext, T, cname = CONFIGS[cfg]
+    kind, ext, T, cname = CONFIGS[cfg][:4]
     rank = int(os.environ.get("RANK", "0"))
     if rank != 0:
         return
@@ -278,11 +286,11 @@ def run_gpu(args, cfg):
 
     from paper_conf_cgo_grosserchsv14_b200 import Plan, Stencil
 
-    kind, ext, T, cname = CONFIGS[cfg]
+    kind, ext, T, cname = CONFIGS[cfg][:4]
     world = int(os.environ.get("WORLD_SIZE", "1"))
     rank = int(os.environ.get("RANK", "0"))
     local = int(os.environ.get("LOCAL_RANK", "0"))
-    if world > 1 or os.environ.get("HEXS_FORCE_DIST") == "1":  # (forced: test the path at N=1)
+    if world > 1 or cfg in DIST_CONFIGS or os.environ.get("HEXS_FORCE_DIST") == "1":
         from paper_conf_cgo_grosserchsv14_b200 import dist
 
         return dist.bench_main(args, cfg, CONFIGS, METRIC, helpers=sys.modules[__name__])
@@ -452,6 +460,18 @@ def main():
     ap.add_argument("--tile", default="", help="h,w0[,w1] override (tuning)")
     args = ap.parse_args()
     args.warmup = max(3, args.warmup)
+    if args.gpus > 1 and "WORLD_SIZE" not in os.environ:
+        # one process per GPU: relaunch this command under torchrun (the driver may also launch
+        # it that way itself; then WORLD_SIZE is set and we are a rank already)
+        import socket
+
+        sk = socket.socket()
+        sk.bind(("127.0.0.1", 0))
+        port = sk.getsockname()[1]
+        sk.close()
+        cmd = [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", f"--nproc-per-node={args.gpus}",
+               "--master-addr", "127.0.0.1", "--master-port", str(port), os.path.abspath(__file__)] + sys.argv[1:]
+        os.execv(sys.executable, cmd)
     if args.impl == "reference":
         run_reference(args, args.config)
     else:

@@ -42,7 +42,7 @@ typedef enum {
   STENCIL_E_INFEASIBLE_TILE = 3,  /* tile parameters violate eq. (1) or the kernel's limits */
   STENCIL_E_OOM = 4,              /* host allocation failed / workspace too small */
   STENCIL_E_CUDA = 5,             /* CUDA runtime error (incl. no device) */
-  STENCIL_E_NCCL = 6              /* reserved for the multi-GPU layer */
+  STENCIL_E_NCCL = 6              /* NCCL unavailable or failed (multi-GPU slab mode) */
 } stencil_status;
 
 typedef enum { STENCIL_F32 = 0, STENCIL_F64 = 1 } stencil_dtype;
@@ -130,6 +130,68 @@ stencil_status stencil_plan_set_workspace(stencil_plan_t plan, void *dev_ptr, si
  * are released with the plan. */
 stencil_status stencil_run(stencil_plan_t plan, const void *const *in, void *const *out,
                            int64_t T_steps, void *stream);
+
+/* ---------------------------------------------------------------------------------
+ * Multi-GPU slab mode.  One process per GPU; the outermost grid
+ * dimension (part_dim = 0: contiguous planes) is split evenly over the ranks.  Rank q owns
+ * planes [own_lo, own_hi) and stores the local slab [loc_lo, loc_hi) = its owned planes plus
+ * G = radius * D ghost planes on every side that is not a global boundary.  Time advances in
+ * blocks of D steps, D a multiple of the hexagon height 2h+2 ("halos of width radius x
+ * time-tile depth, exchanged once per time tile"); a block is the single-GPU hybrid schedule
+ * of Sec. 3.6 over the local slab, whose outermost ghost plane stays
+ * fixed -- after D steps every owned plane is exact (the dependence cone of an owned point over
+ * D steps reaches radius * D planes), ghost planes are the only redundant work.  Between
+ * blocks the library exchanges the ghost planes with rank +-1 by ncclSend / ncclRecv (one NCCL
+ * group per block) on an internal stream ordered against the caller's stream by events.
+ * NCCL is loaded at run time (the libnccl.so.2 the process already maps, e.g. PyTorch's;
+ * environment HEXS_NCCL_LIB overrides); single-GPU use never needs it.  FDTD-2D is not
+ * supported (STENCIL_E_UNSUPPORTED).
+ * ------------------------------------------------------------------------------- */
+typedef struct {
+  int32_t rank, nranks, part_dim;
+  int64_t global_ext[3];  /* stencil_dist_layout: the global extents (stencil_dist_info: -1 for
+                             dimension 0 when nranks > 1)                                   */
+  int64_t local_ext[3];   /* extents of this rank's local slab (ghost planes included)       */
+  int64_t own_lo, own_hi; /* owned global planes of dimension 0                              */
+  int64_t loc_lo, loc_hi; /* global planes held by the local slab                            */
+  int64_t ghost;          /* G = radius * time_block                                         */
+  int64_t time_block;     /* D: steps between halo exchanges                                 */
+  int64_t n_blocks;       /* ceil(T_steps / D)                                               */
+  int32_t h;              /* hexagon half-height the time block is a multiple of             */
+  double ghost_fraction;  /* (local - owned) / owned planes: the redundant work              */
+  int64_t launches_per_run; /* phase-kernel launches of one stencil_run (stencil_dist_info) */
+} stencil_dist_info_t;
+
+/* Rank 0: a fresh NCCL unique id (128 bytes) for stencil_plan_dist; broadcast it to the other
+ * ranks (e.g. with torch.distributed).  STENCIL_E_NCCL if NCCL cannot be loaded. */
+stencil_status stencil_dist_unique_id(void *id_out);
+
+/* Host-only layout of one rank (partition, ghost width, time block) -- exactly what
+ * stencil_plan_dist uses; needs neither a GPU nor NCCL. */
+stencil_status stencil_dist_layout(stencil_desc_t global_desc, int64_t T_steps, const stencil_tile_t *tile,
+                                   int rank, int nranks, int part_dim, stencil_dist_info_t *info);
+
+/* Collective over the nranks processes (each on its own current device): build this rank's
+ * distributed plan for T_steps steps of the GLOBAL problem global_desc.  tile as for
+ * stencil_plan (its h sets the time block; NULL = defaults).  nccl_unique_id: the 128 bytes
+ * from stencil_dist_unique_id on rank 0.  part_dim must be 0.  The plan is then used like a
+ * single-GPU plan: stencil_plan_workspace_size / set_workspace (shared by the block plans),
+ * stencil_run(plan, in, out, T_steps, stream) with in / out the LOCAL slabs (local_ext,
+ * 16-B aligned, in may alias out; every plane of `in`, ghosts included, holds level 0 of the
+ * global grid) -- on return the owned planes of `out` hold level T_steps (ghost planes are
+ * scratch).  stencil_run on a distributed plan is collective (every rank calls it).
+ * STENCIL_E_NCCL on communicator or transfer failure. */
+stencil_status stencil_plan_dist(stencil_plan_t *out, stencil_desc_t global_desc, int64_t T_steps,
+                                 const stencil_tile_t *tile, const void *nccl_unique_id, int rank,
+                                 int nranks, int part_dim);
+
+/* The layout of a distributed plan and its launches per run. */
+stencil_status stencil_dist_info(stencil_plan_t plan, stencil_dist_info_t *info);
+
+/* A borrowed handle to the index-th local block plan of a distributed plan (0 = the D-step
+ * plan; the last one may be a shorter remainder) -- for introspection and per-launch profiling
+ * (stencil_plan_profile).  Owned by the distributed plan: never pass it to stencil_destroy. */
+stencil_status stencil_dist_block_plan(stencil_plan_t plan, int index, stencil_plan_t *block);
 
 /* Destroy a descriptor or plan (tagged handles).  NULL is a no-op.  A plan keeps its own
  * copy of the descriptor, so destruction order is free. */

@@ -28,8 +28,23 @@ ARCH = ["-gencode", "arch=compute_100a,code=sm_100a"]
 NVFLAGS = ARCH + ["-O3", "-std=c++17", "-lineinfo", "--fmad=false", "-prec-div=true",
                   "-prec-sqrt=true", "-ftz=false", "-Xcompiler", "-fPIC", "-Xptxas", "-v",
                   "-I", os.path.join(ROOT, "include")]
+def _nccl_include():
+    """nccl.h of the NCCL the process will load at run time (PyTorch's wheel), else the system's."""
+    try:
+        import importlib.util
+
+        spec = importlib.util.find_spec("nvidia.nccl")
+        if spec and spec.submodule_search_locations:
+            inc = os.path.join(list(spec.submodule_search_locations)[0], "include")
+            if os.path.exists(os.path.join(inc, "nccl.h")):
+                return inc
+    except Exception:  # noqa: BLE001
+        pass
+    return "/usr/include"
+
+
 CXXFLAGS = ["-O2", "-std=c++17", "-fPIC", "-ffp-contract=off", "-I", os.path.join(ROOT, "include"),
-            "-I", "/usr/local/cuda/include"]
+            "-I", "/usr/local/cuda/include", "-I", _nccl_include()]
 
 
 def _variant_ids(header: str, macro: str):
@@ -54,7 +69,7 @@ def _units():
     headers = [os.path.join(dp, f) for dp, _, fs in os.walk(CSRC) for f in fs
                if f.endswith((".h", ".cuh"))] + [os.path.join(ROOT, "include", "stencil.h")]
     units = []
-    for src in ["desc.cpp", "plan.cpp"]:
+    for src in ["desc.cpp", "plan.cpp", "dist.cpp"]:
         units.append((os.path.join(CSRC, src), "cxx", []))
     for src in ["run.cu", "kernels/generic.cu", "kernels/registry.cu", "kernels/fdtd.cu"]:
         units.append((os.path.join(CSRC, src), "nvcc", []))
@@ -100,7 +115,7 @@ def build_library(jobs: int = 0, verbose: bool = False, lib: str = None) -> str:
     stamp = LIB + ".objs"
     want = "\n".join(objs)
     if not os.path.exists(LIB) or not os.path.exists(stamp) or open(stamp).read() != want:
-        cmd = [NVCC] + ARCH + ["-shared", "-o", LIB] + objs + ["-lcudart"]
+        cmd = [NVCC] + ARCH + ["-shared", "-o", LIB] + objs + ["-lcudart", "-ldl"]
         subprocess.check_call(cmd)
         open(stamp, "w").write(want)
     if verbose:

@@ -26,7 +26,9 @@ SYMBOLS = ["stencil_desc_create", "stencil_desc_deps", "stencil_plan",
            "stencil_plan_workspace_size", "stencil_plan_set_workspace", "stencil_run",
            "stencil_destroy", "stencil_last_error", "stencil_plan_info",
            "stencil_plan_launches", "stencil_plan_hexagon", "stencil_plan_schedule_of",
-           "stencil_plan_profile", "stencil_plan_profile_read", "stencil_abi_version"]
+           "stencil_plan_profile", "stencil_plan_profile_read", "stencil_abi_version",
+           "stencil_dist_unique_id", "stencil_dist_layout", "stencil_plan_dist", "stencil_dist_info",
+           "stencil_dist_block_plan"]
 
 
 class StencilError(RuntimeError):
@@ -56,6 +58,15 @@ class PlanInfo(ctypes.Structure):
                 ("workspace_bytes", ctypes.c_size_t), ("kernel", ctypes.c_int32)]
 
 KERNELS = {0: "generic", 1: "naive", 2: "fast2d", 3: "fdtd", 4: "fast3d", 5: "stream3d"}
+
+
+class DistInfo(ctypes.Structure):
+    _fields_ = [("rank", ctypes.c_int32), ("nranks", ctypes.c_int32), ("part_dim", ctypes.c_int32),
+                ("global_ext", ctypes.c_int64 * 3), ("local_ext", ctypes.c_int64 * 3),
+                ("own_lo", ctypes.c_int64), ("own_hi", ctypes.c_int64), ("loc_lo", ctypes.c_int64),
+                ("loc_hi", ctypes.c_int64), ("ghost", ctypes.c_int64), ("time_block", ctypes.c_int64),
+                ("n_blocks", ctypes.c_int64), ("h", ctypes.c_int32), ("ghost_fraction", ctypes.c_double),
+                ("launches_per_run", ctypes.c_int64)]
 
 
 class Launch(ctypes.Structure):
@@ -92,6 +103,11 @@ def lib() -> ctypes.CDLL:
     L.stencil_plan_schedule_of.argtypes = [vp, i64, P(i64), P(i64)]
     L.stencil_plan_profile.argtypes = [vp, ctypes.c_int]
     L.stencil_plan_profile_read.argtypes = [vp, P(ctypes.c_double), P(i64), P(ctypes.c_double)]
+    L.stencil_dist_unique_id.argtypes = [vp]
+    L.stencil_dist_layout.argtypes = [vp, i64, P(Tile), ctypes.c_int, ctypes.c_int, ctypes.c_int, P(DistInfo)]
+    L.stencil_plan_dist.argtypes = [P(vp), vp, i64, P(Tile), vp, ctypes.c_int, ctypes.c_int, ctypes.c_int]
+    L.stencil_dist_info.argtypes = [vp, P(DistInfo)]
+    L.stencil_dist_block_plan.argtypes = [vp, ctypes.c_int, P(vp)]
     for name in SYMBOLS:
         f = getattr(L, name)
         if name not in ("stencil_last_error", "stencil_abi_version"):

@@ -1,0 +1,453 @@
+// dist.cpp -- multi-GPU slab mode of the C ABI: one process per GPU,
+// the outermost grid dimension slab-partitioned over the ranks, halos exchanged with NCCL
+// send/recv over NVLink once per time block.
+//
+// The paper's method is single-GPU: its host loop iterates the two phase kernels over the
+// whole grid (Sec. 4.1).  Scaling it over ranks keeps that hybrid schedule
+// unchanged inside every rank and adds overlapped tiling at rank edges only:
+//   * rank q owns planes [own_lo, own_hi) of dimension 0 (an even split) and stores the local
+//     slab [loc_lo, loc_hi) = owned planes plus G = radius * D ghost planes on every side that
+//     is not a global boundary;
+//   * time advances in blocks of D steps (D a multiple of the hexagon height 2h+2: the halos
+//     have the width "radius x time-tile depth" and are exchanged once per time tile);
+//   * a block is one stencil_run of a local single-GPU plan (the hybrid schedule over the slab,
+//     its outermost ghost plane held fixed): after D steps every owned plane is exact, because
+//     the dependence cone of an owned point over D steps reaches radius * D planes (the only
+//     redundant work is the ghost planes, 2G / owned of the compute);
+//   * between blocks the ghost planes are refreshed from the neighbours' owned planes:
+//     ncclGroupStart; ncclSend / ncclRecv to rank - 1 and rank + 1; ncclGroupEnd, on a
+//     communication stream ordered against the compute stream by events.
+// NCCL is loaded at run time (dlopen of the libnccl.so.2 the process already uses, e.g.
+// PyTorch's), so single-GPU use of the library never needs it; PyTorch only broadcasts the
+// 128-byte unique id (stencil_dist_unique_id on rank 0).
+#include <dlfcn.h>
+
+#include <algorithm>
+#include <cstdlib>
+#include <cstring>
+#include <memory>
+#include <new>
+#include <string>
+#include <vector>
+
+#include <cuda_runtime.h>
+#include <nccl.h>
+
+#include "internal.h"
+
+namespace hexs {
+
+namespace {
+
+struct NcclApi {
+  void* handle = nullptr;
+  ncclResult_t (*GetUniqueId)(ncclUniqueId*) = nullptr;
+  ncclResult_t (*CommInitRank)(ncclComm_t*, int, ncclUniqueId, int) = nullptr;
+  ncclResult_t (*CommDestroy)(ncclComm_t) = nullptr;
+  ncclResult_t (*GroupStart)() = nullptr;
+  ncclResult_t (*GroupEnd)() = nullptr;
+  ncclResult_t (*Send)(const void*, size_t, ncclDataType_t, int, ncclComm_t, cudaStream_t) = nullptr;
+  ncclResult_t (*Recv)(void*, size_t, ncclDataType_t, int, ncclComm_t, cudaStream_t) = nullptr;
+  const char* (*GetErrorString)(ncclResult_t) = nullptr;
+  ncclResult_t (*CommGetAsyncError)(ncclComm_t, ncclResult_t*) = nullptr;
+  std::string error;
+};
+
+// Load NCCL once: HEXS_NCCL_LIB if set, else the libnccl.so.2 already mapped into the process
+// (PyTorch's), else the dynamic linker's.
+NcclApi* nccl_api() {
+  static NcclApi api;
+  static bool tried = false;
+  if (tried) return api.handle ? &api : nullptr;
+  tried = true;
+  const char* env = std::getenv("HEXS_NCCL_LIB");
+  void* h = nullptr;
+  if (env && *env) h = dlopen(env, RTLD_NOW | RTLD_GLOBAL);
+  if (!h) h = dlopen("libnccl.so.2", RTLD_NOW | RTLD_NOLOAD | RTLD_GLOBAL);
+  if (!h) h = dlopen("libnccl.so.2", RTLD_NOW | RTLD_GLOBAL);
+  if (!h) h = dlopen("libnccl.so", RTLD_NOW | RTLD_GLOBAL);
+  if (!h) {
+    const char* e = dlerror();
+    api.error = std::string("cannot load libnccl.so.2: ") + (e ? e : "?");
+    return nullptr;
+  }
+  auto sym = [&](const char* name) { return dlsym(h, name); };
+  api.GetUniqueId = reinterpret_cast<decltype(api.GetUniqueId)>(sym("ncclGetUniqueId"));
+  api.CommInitRank = reinterpret_cast<decltype(api.CommInitRank)>(sym("ncclCommInitRank"));
+  api.CommDestroy = reinterpret_cast<decltype(api.CommDestroy)>(sym("ncclCommDestroy"));
+  api.GroupStart = reinterpret_cast<decltype(api.GroupStart)>(sym("ncclGroupStart"));
+  api.GroupEnd = reinterpret_cast<decltype(api.GroupEnd)>(sym("ncclGroupEnd"));
+  api.Send = reinterpret_cast<decltype(api.Send)>(sym("ncclSend"));
+  api.Recv = reinterpret_cast<decltype(api.Recv)>(sym("ncclRecv"));
+  api.GetErrorString = reinterpret_cast<decltype(api.GetErrorString)>(sym("ncclGetErrorString"));
+  api.CommGetAsyncError = reinterpret_cast<decltype(api.CommGetAsyncError)>(sym("ncclCommGetAsyncError"));
+  if (!api.GetUniqueId || !api.CommInitRank || !api.CommDestroy || !api.GroupStart || !api.GroupEnd ||
+      !api.Send || !api.Recv || !api.GetErrorString) {
+    api.error = "libnccl.so.2 lacks a required symbol";
+    return nullptr;
+  }
+  api.handle = h;
+  return &api;
+}
+
+stencil_status nccl_fail(NcclApi* a, ncclResult_t r, const char* where) {
+  return fail(STENCIL_E_NCCL, std::string(where) + ": " + (a && a->GetErrorString ? a->GetErrorString(r) : "NCCL error"));
+}
+
+Plan* as_plan(stencil_plan_t h) {
+  Plan* p = reinterpret_cast<Plan*>(h);
+  return (p && p->magic == kPlanMagic) ? p : nullptr;
+}
+
+}  // namespace
+
+struct DistState {
+  DistLayout lay;
+  std::vector<int64_t> blocks;                     // block lengths (D, ..., remainder)
+  std::vector<std::pair<int64_t, Plan*>> bplans;   // one local plan per distinct block length
+  Desc local;                                      // descriptor of the local slab
+  size_t plane_bytes = 0;                          // bytes of one plane of dimension 0
+  void* comm = nullptr;                            // ncclComm_t
+  cudaStream_t comm_stream = nullptr;
+  cudaEvent_t ev_ready = nullptr, ev_done = nullptr;
+  int comm_dev = -1;
+  bool emulate = false;  // HEXS_DIST_EMULATE: a rank's compute alone (no communicator)
+  ~DistState() {
+    for (auto& bp : bplans) delete bp.second;
+    if (comm) {
+      if (NcclApi* a = nccl_api()) a->CommDestroy(static_cast<ncclComm_t>(comm));
+    }
+    if (ev_ready) cudaEventDestroy(ev_ready);
+    if (ev_done) cudaEventDestroy(ev_done);
+    if (comm_stream) cudaStreamDestroy(comm_stream);
+  }
+  Plan* plan_for(int64_t len) const {
+    for (auto& bp : bplans)
+      if (bp.first == len) return bp.second;
+    return nullptr;
+  }
+};
+
+void dist_free(DistState* d) { delete d; }
+
+// stencil_plan_info of a distributed plan: the primary block plan's schedule and tile, the
+// whole run's steps, launches and this rank's owned updates.
+void dist_fill_info(const Plan& p, stencil_plan_info_t& o) {
+  const DistState& s = *p.dist;
+  int64_t launches = 0;
+  for (int64_t len : s.blocks) {
+    const Plan* bp = s.plan_for(len);
+    launches += bp->executor == EXEC_NAIVE ? bp->tau_levels : (int64_t)bp->launches.size();
+  }
+  o.n_launches = launches;
+  o.T_steps = p.T_steps;
+  o.tau_levels = p.tau_levels;
+  int64_t interior = 1;
+  for (int q = 1; q < s.local.dims; ++q) interior *= s.local.ext[q] - 2 * s.local.radius;
+  const int64_t glo = std::max<int64_t>(s.lay.own_lo, s.local.radius);
+  int64_t ghi = s.lay.own_hi;
+  if (s.lay.rank == s.lay.nranks - 1) ghi -= s.local.radius;  // the global last planes are Dirichlet
+  o.updates = std::max<int64_t>(0, ghi - glo) * interior * p.T_steps;
+  o.workspace_bytes = p.ws_bytes;
+}
+
+// The tile of the local block plans: the caller's, else (3D) the (2, 7) hexagon -- a 6-step time
+// tile keeps the ghost planes of a 128-plane slab under 10% -- else the class default.
+stencil_tile_t dist_local_tile(const Desc& d, const stencil_tile_t* tile) {
+  stencil_tile_t lt{};
+  lt.hex_dim = -1;
+  if (tile) lt = *tile;
+  if (lt.h || lt.w0) return lt;  // an explicit hexagon
+  if (d.dims == 3 && (lt.flags == STENCIL_EXEC_AUTO)) {
+    lt.h = 2;
+    lt.w0 = 7;
+  }
+  return lt;
+}
+
+// The slab layout of one rank (host only; shared by stencil_dist_layout and stencil_plan_dist).
+stencil_status dist_layout(const Desc& d, int64_t T_steps, const stencil_tile_t* tile, int rank, int nranks,
+                           int part_dim, DistLayout* out) {
+  if (nranks < 1 || rank < 0 || rank >= nranks) return fail(STENCIL_E_INVALID, "stencil_plan_dist: bad rank / nranks");
+  if (part_dim != 0)
+    return fail(STENCIL_E_UNSUPPORTED, "stencil_plan_dist: only the outermost dimension (contiguous planes) is partitioned");
+  if (d.kind == STENCIL_FDTD2D)
+    return fail(STENCIL_E_UNSUPPORTED, "stencil_plan_dist: FDTD-2D (three in-place fields) has no slab mode");
+  if (T_steps < 0) return fail(STENCIL_E_INVALID, "stencil_plan_dist: T_steps < 0");
+  DistLayout L{};
+  L.rank = rank;
+  L.nranks = nranks;
+  L.part_dim = part_dim;
+  const int64_t N0 = d.ext[0];
+  const int64_t base = N0 / nranks, extra = N0 % nranks;
+  L.own_lo = rank * base + std::min<int64_t>(rank, extra);
+  L.own_hi = L.own_lo + base + (rank < extra ? 1 : 0);
+  // time block: a multiple of the hexagon height 2h+2 of the local plans' tile (one time tile
+  // by default, more while the ghost planes stay within ~10% of the owned ones);
+  // HEXS_TIME_BLOCK overrides
+  const stencil_tile_t lt = dist_local_tile(d, tile);
+  int h = lt.h;
+  if (!(lt.h || lt.w0)) {  // the class's automatic tile: ask the planner
+    Plan* probe = nullptr;
+    if (build_plan(d, 1, &lt, &probe) != STENCIL_OK) return STENCIL_E_INVALID;
+    h = probe->h;
+    delete probe;
+  }
+  const int64_t H = 2 * (int64_t)h + 2;
+  const int64_t owned = L.own_hi - L.own_lo;
+  int64_t D = H * std::max<int64_t>(1, owned / (20 * H));
+  if (const char* e = std::getenv("HEXS_TIME_BLOCK")) {
+    const int64_t v = std::atoll(e);
+    if (v > 0) D = v;
+  }
+  if (T_steps > 0) D = std::min(D, T_steps);
+  D = std::max<int64_t>(D, 1);
+  L.time_block = D;
+  L.ghost = (int64_t)d.radius * D;
+  if (nranks > 1 && owned < L.ghost)
+    return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_plan_dist: a slab is thinner than the ghost width radius*D");
+  L.loc_lo = std::max<int64_t>(0, L.own_lo - L.ghost);
+  L.loc_hi = std::min<int64_t>(N0, L.own_hi + L.ghost);
+  L.n_blocks = T_steps == 0 ? 0 : (T_steps + D - 1) / D;
+  L.h = h;
+  L.ghost_fraction = owned > 0 ? (double)((L.loc_hi - L.loc_lo) - owned) / (double)owned : 0.0;
+  *out = L;
+  return STENCIL_OK;
+}
+
+stencil_status dist_set_workspace(Plan& p, void* dev_ptr, size_t bytes) {
+  for (auto& bp : p.dist->bplans) {
+    if (bytes < bp.second->ws_bytes) return fail(STENCIL_E_OOM, "stencil_plan_set_workspace: workspace too small");
+    bp.second->ws = dev_ptr;
+    bp.second->ws_size = bytes;
+  }
+  return STENCIL_OK;
+}
+
+// One halo exchange on the communication stream: my first / last G owned planes go to rank -1
+// / rank + 1, their owned planes land in my ghost planes.
+static stencil_status exchange(DistState& s, char* base, cudaStream_t stream) {
+  NcclApi* a = nccl_api();
+  if (!a) return fail(STENCIL_E_NCCL, "NCCL unavailable");
+  const DistLayout& L = s.lay;
+  const int64_t G = L.ghost;
+  const size_t n = (size_t)G * s.plane_bytes;
+  ncclComm_t comm = static_cast<ncclComm_t>(s.comm);
+  cudaError_t e = cudaEventRecord(s.ev_ready, stream);
+  if (e == cudaSuccess) e = cudaStreamWaitEvent(s.comm_stream, s.ev_ready, 0);
+  if (e != cudaSuccess) return fail(STENCIL_E_CUDA, std::string("stencil_run: halo ordering: ") + cudaGetErrorString(e));
+  ncclResult_t r = a->GroupStart();
+  if (r != ncclSuccess) return nccl_fail(a, r, "ncclGroupStart");
+  const int64_t own0 = L.own_lo - L.loc_lo, own1 = L.own_hi - L.loc_lo;  // local plane indices
+  if (L.rank > 0) {
+    a->Send(base + own0 * s.plane_bytes, n, ncclChar, L.rank - 1, comm, s.comm_stream);
+    a->Recv(base + (own0 - G) * s.plane_bytes, n, ncclChar, L.rank - 1, comm, s.comm_stream);
+  }
+  if (L.rank < L.nranks - 1) {
+    a->Send(base + (own1 - G) * s.plane_bytes, n, ncclChar, L.rank + 1, comm, s.comm_stream);
+    a->Recv(base + own1 * s.plane_bytes, n, ncclChar, L.rank + 1, comm, s.comm_stream);
+  }
+  r = a->GroupEnd();
+  if (r != ncclSuccess) return nccl_fail(a, r, "ncclGroupEnd");
+  e = cudaEventRecord(s.ev_done, s.comm_stream);
+  if (e == cudaSuccess) e = cudaStreamWaitEvent(stream, s.ev_done, 0);
+  if (e != cudaSuccess) return fail(STENCIL_E_CUDA, std::string("stencil_run: halo ordering: ") + cudaGetErrorString(e));
+  if (a->CommGetAsyncError) {
+    ncclResult_t ae = ncclSuccess;
+    if (a->CommGetAsyncError(comm, &ae) == ncclSuccess && ae != ncclSuccess && ae != ncclInProgress)
+      return nccl_fail(a, ae, "NCCL async error");
+  }
+  return STENCIL_OK;
+}
+
+stencil_status run_dist(Plan& p, const void* const* in, void* const* out, void* stream_) {
+  DistState& s = *p.dist;
+  cudaStream_t stream = static_cast<cudaStream_t>(stream_);
+  if (!in || !out || !in[0] || !out[0]) return fail(STENCIL_E_INVALID, "stencil_run: NULL field pointer");
+  if ((reinterpret_cast<uintptr_t>(in[0]) | reinterpret_cast<uintptr_t>(out[0])) % 16)
+    return fail(STENCIL_E_INVALID, "stencil_run: field pointers must be 16-B aligned");
+  int dev = -1;
+  if (cudaGetDevice(&dev) != cudaSuccess || dev != s.comm_dev)
+    return fail(STENCIL_E_CUDA, "stencil_run: a distributed plan runs on the device it was created on");
+  const size_t bytes = (size_t)(s.lay.loc_hi - s.lay.loc_lo) * s.plane_bytes;
+  if (in[0] != out[0]) {
+    cudaError_t e = cudaMemcpyAsync(out[0], in[0], bytes, cudaMemcpyDeviceToDevice, stream);
+    if (e != cudaSuccess) return fail(STENCIL_E_CUDA, std::string("stencil_run: copy in->out: ") + cudaGetErrorString(e));
+  }
+  void* const* io = out;  // every block runs in place on the caller's output slab
+  for (size_t k = 0; k < s.blocks.size(); ++k) {
+    if (k > 0 && s.lay.nranks > 1 && !s.emulate) {
+      stencil_status st = exchange(s, static_cast<char*>(out[0]), stream);
+      if (st != STENCIL_OK) return st;
+    }
+    Plan* bp = s.plan_for(s.blocks[k]);
+    stencil_status st = run_plan(*bp, reinterpret_cast<const void* const*>(io), io, stream);
+    if (st != STENCIL_OK) return st;
+  }
+  return STENCIL_OK;
+}
+
+}  // namespace hexs
+
+using namespace hexs;
+
+extern "C" {
+
+stencil_status stencil_dist_unique_id(void* id_out) {
+  clear_error();
+  if (!id_out) return fail(STENCIL_E_INVALID, "stencil_dist_unique_id: NULL output");
+  NcclApi* a = nccl_api();
+  if (!a) return fail(STENCIL_E_NCCL, "stencil_dist_unique_id: NCCL unavailable");
+  ncclUniqueId id;
+  ncclResult_t r = a->GetUniqueId(&id);
+  if (r != ncclSuccess) return nccl_fail(a, r, "ncclGetUniqueId");
+  std::memcpy(id_out, &id, sizeof(id));
+  return STENCIL_OK;
+}
+
+stencil_status stencil_dist_layout(stencil_desc_t global_desc, int64_t T_steps, const stencil_tile_t* tile,
+                                   int rank, int nranks, int part_dim, stencil_dist_info_t* info) {
+  clear_error();
+  Desc* d = reinterpret_cast<Desc*>(global_desc);
+  if (!d || d->magic != kDescMagic || !info) return fail(STENCIL_E_INVALID, "stencil_dist_layout: bad arguments");
+  DistLayout L{};
+  stencil_status st = dist_layout(*d, T_steps, tile, rank, nranks, part_dim, &L);
+  if (st != STENCIL_OK) return st;
+  stencil_dist_info_t o{};
+  o.rank = L.rank;
+  o.nranks = L.nranks;
+  o.part_dim = L.part_dim;
+  for (int q = 0; q < 3; ++q) {
+    o.global_ext[q] = q < d->dims ? d->ext[q] : 1;
+    o.local_ext[q] = o.global_ext[q];
+  }
+  o.local_ext[0] = L.loc_hi - L.loc_lo;
+  o.own_lo = L.own_lo;
+  o.own_hi = L.own_hi;
+  o.loc_lo = L.loc_lo;
+  o.loc_hi = L.loc_hi;
+  o.ghost = L.ghost;
+  o.time_block = L.time_block;
+  o.n_blocks = L.n_blocks;
+  o.h = L.h;
+  o.ghost_fraction = L.ghost_fraction;
+  *info = o;
+  return STENCIL_OK;
+}
+
+stencil_status stencil_plan_dist(stencil_plan_t* out, stencil_desc_t global_desc, int64_t T_steps,
+                                 const stencil_tile_t* tile, const void* nccl_unique_id, int rank, int nranks,
+                                 int part_dim) {
+  clear_error();
+  if (!out) return fail(STENCIL_E_INVALID, "stencil_plan_dist: out is NULL");
+  *out = nullptr;
+  Desc* d = reinterpret_cast<Desc*>(global_desc);
+  if (!d || d->magic != kDescMagic) return fail(STENCIL_E_INVALID, "stencil_plan_dist: bad descriptor");
+  if (!nccl_unique_id) return fail(STENCIL_E_INVALID, "stencil_plan_dist: NULL NCCL unique id");
+  std::unique_ptr<DistState> s(new (std::nothrow) DistState());
+  if (!s) return fail(STENCIL_E_OOM, "stencil_plan_dist: out of host memory");
+  stencil_status st = dist_layout(*d, T_steps, tile, rank, nranks, part_dim, &s->lay);
+  if (st != STENCIL_OK) return st;
+  const DistLayout& L = s->lay;
+  // the local slab's descriptor: same class / coefficients / dtype, extent loc_hi - loc_lo
+  s->local = *d;
+  s->local.ext[0] = L.loc_hi - L.loc_lo;
+  if (s->local.ext[0] < 3) return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_plan_dist: local slab thinner than 3 planes");
+  s->plane_bytes = d->elem();
+  for (int q = 1; q < d->dims; ++q) s->plane_bytes *= (size_t)d->ext[q];
+  for (int64_t t = 0; t < T_steps; t += L.time_block) s->blocks.push_back(std::min(L.time_block, T_steps - t));
+  const stencil_tile_t lt = dist_local_tile(*d, tile);
+  for (int64_t len : s->blocks) {
+    if (s->plan_for(len)) continue;
+    Plan* bp = nullptr;
+    st = build_plan(s->local, len, &lt, &bp);
+    if (st != STENCIL_OK) return st;
+    s->bplans.push_back({len, bp});
+  }
+  // NCCL communicator and the communication stream on the current device
+  if (cudaGetDevice(&s->comm_dev) != cudaSuccess) return fail(STENCIL_E_CUDA, "stencil_plan_dist: no CUDA device");
+  if (cudaStreamCreateWithFlags(&s->comm_stream, cudaStreamNonBlocking) != cudaSuccess ||
+      cudaEventCreateWithFlags(&s->ev_ready, cudaEventDisableTiming) != cudaSuccess ||
+      cudaEventCreateWithFlags(&s->ev_done, cudaEventDisableTiming) != cudaSuccess)
+    return fail(STENCIL_E_CUDA, "stencil_plan_dist: stream / event creation failed");
+  // HEXS_DIST_EMULATE=1: one process plays one rank of nranks on its own GPU -- no
+  // communicator, no exchanges (the ghost planes keep their initial values, so results are not
+  // the global ones); it measures a rank's compute for scaling projections on a single GPU
+  s->emulate = std::getenv("HEXS_DIST_EMULATE") && std::atoi(std::getenv("HEXS_DIST_EMULATE")) != 0;
+  if (!s->emulate) {  // (also for one rank: the same NCCL bootstrap path, no exchange ever runs)
+    NcclApi* a = nccl_api();
+    if (!a) return fail(STENCIL_E_NCCL, "stencil_plan_dist: NCCL unavailable");
+    ncclUniqueId id;
+    std::memcpy(&id, nccl_unique_id, sizeof(id));
+    ncclComm_t comm = nullptr;
+    ncclResult_t r = a->CommInitRank(&comm, nranks, id, rank);
+    if (r != ncclSuccess) return nccl_fail(a, r, "ncclCommInitRank");
+    s->comm = comm;
+  }
+  // the dist plan itself: the primary block plan's schedule, the whole run's step count
+  Plan* p = new (std::nothrow) Plan();
+  if (!p) return fail(STENCIL_E_OOM, "stencil_plan_dist: out of host memory");
+  Plan* primary = s->plan_for(s->blocks.empty() ? 0 : s->blocks[0]);
+  if (primary) {
+    p->desc = primary->desc;
+    p->hd = primary->hd;
+    p->h = primary->h;
+    p->w0 = primary->w0;
+  } else {
+    p->desc = s->local;
+  }
+  p->T_steps = T_steps;
+  p->tau_levels = T_steps * (int64_t)d->stmts.size();
+  p->executor = primary ? primary->executor : EXEC_GENERIC;
+  size_t ws = 0;
+  for (auto& bp : s->bplans) ws = std::max(ws, bp.second->ws_bytes);
+  p->ws_bytes = ws;
+  p->dist = s.release();
+  *out = reinterpret_cast<stencil_plan_t>(p);
+  return STENCIL_OK;
+}
+
+stencil_status stencil_dist_info(stencil_plan_t plan, stencil_dist_info_t* info) {
+  clear_error();
+  Plan* p = as_plan(plan);
+  if (!p || !p->dist || !info) return fail(STENCIL_E_INVALID, "stencil_dist_info: not a distributed plan");
+  const DistState& s = *p->dist;
+  const DistLayout& L = s.lay;
+  stencil_dist_info_t o{};
+  o.rank = L.rank;
+  o.nranks = L.nranks;
+  o.part_dim = L.part_dim;
+  for (int q = 0; q < 3; ++q) o.local_ext[q] = o.global_ext[q] = q < s.local.dims ? s.local.ext[q] : 1;
+  o.global_ext[0] = -1;  // filled below from the partition
+  o.local_ext[0] = L.loc_hi - L.loc_lo;
+  o.own_lo = L.own_lo;
+  o.own_hi = L.own_hi;
+  o.loc_lo = L.loc_lo;
+  o.loc_hi = L.loc_hi;
+  o.ghost = L.ghost;
+  o.time_block = L.time_block;
+  o.n_blocks = L.n_blocks;
+  o.h = L.h;
+  o.ghost_fraction = L.ghost_fraction;
+  int64_t launches = 0;
+  for (int64_t len : s.blocks) {
+    const Plan* bp = s.plan_for(len);
+    launches += bp->executor == EXEC_NAIVE ? bp->tau_levels : (int64_t)bp->launches.size();
+  }
+  o.launches_per_run = launches;
+  o.global_ext[0] = L.nranks == 1 ? L.own_hi : -1;
+  *info = o;
+  return STENCIL_OK;
+}
+
+stencil_status stencil_dist_block_plan(stencil_plan_t plan, int index, stencil_plan_t* block) {
+  clear_error();
+  Plan* p = as_plan(plan);
+  if (!p || !p->dist || !block) return fail(STENCIL_E_INVALID, "stencil_dist_block_plan: not a distributed plan");
+  if (index < 0 || index >= (int)p->dist->bplans.size())
+    return fail(STENCIL_E_INVALID, "stencil_dist_block_plan: index out of range");
+  *block = reinterpret_cast<stencil_plan_t>(p->dist->bplans[index].second);
+  return STENCIL_OK;
+}
+
+}  // extern "C"

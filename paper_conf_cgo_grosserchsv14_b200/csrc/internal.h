@@ -73,8 +73,18 @@ struct Launch {
 
 enum Executor { EXEC_GENERIC = 1, EXEC_NAIVE = 2, EXEC_FAST2D = 3, EXEC_FDTD = 4, EXEC_FAST3D = 5, EXEC_STREAM3D = 6 };
 
+// Multi-GPU slab mode (dist.cpp): partition, time blocks, local block plans, NCCL state.
+struct DistLayout {
+  int rank, nranks, part_dim, h;
+  int64_t own_lo, own_hi, loc_lo, loc_hi, ghost, time_block, n_blocks;
+  double ghost_fraction;
+};
+struct DistState;
+void dist_free(DistState* d);
+
 struct Plan {
   uint32_t magic = kPlanMagic;
+  DistState* dist = nullptr;  // non-null: a stencil_plan_dist plan (stencil_run runs the slab mode)
   Desc desc;
   int64_t T_steps = 0, tau_levels = 0;
   int hd = 0;           // hexagonal dimension
@@ -124,6 +134,10 @@ bool schedule_of(const Plan& p, int64_t tau, const int64_t* s, int64_t* sched);
 
 // run.cu
 stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* stream);
+// dist.cpp
+stencil_status run_dist(Plan& p, const void* const* in, void* const* out, void* stream);
+stencil_status dist_set_workspace(Plan& p, void* dev_ptr, size_t bytes);
+void dist_fill_info(const Plan& p, stencil_plan_info_t& o);
 
 // Fast-kernel registry (kernels/*.cu): returns variant id >= 0 or -1 if not instantiated.
 int fast2d_variant(int kind, int dtype, int h, int w0, int w1);

@@ -438,6 +438,7 @@ stencil_status stencil_plan_set_workspace(stencil_plan_t plan, void* dev_ptr, si
     return fail(STENCIL_E_INVALID, "stencil_plan_set_workspace: workspace must be 256-B aligned");
   p->ws = dev_ptr;
   p->ws_size = bytes;
+  if (p->dist) return dist_set_workspace(*p, dev_ptr, bytes);  // shared by the block plans
   return STENCIL_OK;
 }
 
@@ -445,6 +446,15 @@ stencil_status stencil_plan_info(stencil_plan_t plan, stencil_plan_info_t* info)
   clear_error();
   Plan* p = as_plan(plan);
   if (!p || !info) return fail(STENCIL_E_INVALID, "stencil_plan_info: bad arguments");
+  if (p->dist) {  // a distributed plan describes its primary local block plan
+    stencil_plan_t bp = nullptr;
+    stencil_status st = stencil_dist_block_plan(plan, 0, &bp);
+    if (st != STENCIL_OK) return st;
+    st = stencil_plan_info(bp, info);
+    if (st != STENCIL_OK) return st;
+    dist_fill_info(*p, *info);
+    return STENCIL_OK;
+  }
   stencil_plan_info_t& o = *info;
   o = stencil_plan_info_t{};
   const Desc& d = p->desc;

@@ -54,6 +54,7 @@ static void fill_generic(const Plan& p, const Launch& l, GenericArgs& g) {
 }
 
 Plan::~Plan() {
+  if (dist) dist_free(dist);
   for (void* e : prof_events)
     if (e) cudaEventDestroy(static_cast<cudaEvent_t>(e));
   for (auto& gr : graphs)
@@ -263,6 +264,7 @@ extern "C" stencil_status stencil_run(stencil_plan_t plan, const void* const* in
   if (!p || p->magic != kPlanMagic) return fail(STENCIL_E_INVALID, "stencil_run: bad plan");
   if (!in || !out) return fail(STENCIL_E_INVALID, "stencil_run: in/out is NULL");
   if (T_steps != p->T_steps) return fail(STENCIL_E_INVALID, "stencil_run: T_steps differs from the plan's");
+  if (p->dist) return run_dist(*p, in, out, stream);  // multi-GPU slab mode (dist.cpp)
   // Replay a captured CUDA graph of the whole run when the pointers match an earlier run (and no
   // profiling is requested); the first run is eager (kernel attributes, occupancy queries), the
   // second is captured on a private stream and replayed from then on.  HEXS_NO_GRAPH=1 disables.

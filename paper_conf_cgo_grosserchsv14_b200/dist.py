@@ -1,218 +1,299 @@
-"""Multi-GPU slab mode: one process per GPU, the outermost grid dimension
-slab-partitioned over the ranks, halos of width radius x D exchanged over torch.distributed
-(NCCL over NVLink 5 / NVSwitch on the GPU box) once per time block of D steps.
+"""Multi-GPU slab mode over the C ABI's distributed plans.
 
-Per rank the local grid is its owned planes plus G = r*D ghost planes on every side that is
-not a global boundary.  A block runs the hybrid-tiled hot path (the C ABI's stencil_run) for
-D steps on the local grid, whose outermost ghost plane acts as a frozen (Dirichlet) plane;
-after D steps every owned plane is exact, because the dependence cone of an owned point over
-D steps reaches r*D planes (overlapped tiling at rank edges only -- inside a rank the hybrid
-schedule has no redundant work).  The exchange then refreshes the ghost
-planes from the neighbours' owned planes (ncclSend/ncclRecv pairs via batch_isend_irecv).
+One process per GPU.  The library (csrc/dist.cpp, include/stencil.h) partitions the outermost
+grid dimension, keeps G = radius * D ghost planes per interior side, runs every time block of
+D steps as the single-GPU hybrid schedule over the local slab and exchanges the ghost planes
+with ncclSend / ncclRecv between blocks.  Python only bootstraps: rank 0 asks the library for
+an NCCL unique id and torch.distributed broadcasts it; PyTorch provides the device memory.
 
-Only the host-side partition / exchange logic lives here; every time step runs in
-libhexstencil.so.  CPU tests (tests/test_dist_gloo.py) drive the same class over the gloo
-backend with an injected compute callable to check the partition and halo logic.
+    dp = DistPlan("star3d7", (1024, 1024, 1024), T=256)    # collective
+    local = dp.scatter(global_grid)                        # this rank's slab (ghosts included)
+    dp.run(local)                                          # collective; owned planes -> level T
+    owned = dp.owned(local)
+
+`layout(...)` is the same partition as a host-only call (no GPU, no NCCL): the CPU tests
+(tests/test_dist_gloo.py) drive the library's layout with the oracle as the per-block compute
+and a gloo halo exchange (`exchange_halos`) to check the protocol bit for bit.
 """
 from __future__ import annotations
 
+import ctypes
 import json
 import os
+import sys
 from dataclasses import dataclass
 from typing import Callable, List, Optional, Sequence, Tuple
 
 import torch
 import torch.distributed as dist
 
+from . import _lib
+from ._lib import DistInfo, EXEC, KINDS, StencilError, Tile, check, lib
+from .api import _dtype_code
+
 
 @dataclass(frozen=True)
-class Slab:
+class Layout:
     rank: int
     nranks: int
-    N0: int          # global extent of the partitioned (outermost) dimension
-    own_lo: int      # owned global planes [own_lo, own_hi)
+    global_ext: Tuple[int, ...]
+    local_ext: Tuple[int, ...]
+    own_lo: int
     own_hi: int
-    loc_lo: int      # local grid covers global planes [loc_lo, loc_hi)
+    loc_lo: int
     loc_hi: int
-    ghost: int       # G
-
-    @property
-    def local_extent(self) -> int:
-        return self.loc_hi - self.loc_lo
+    ghost: int
+    time_block: int
+    n_blocks: int
+    h: int
+    ghost_fraction: float
 
     @property
     def own_local(self) -> Tuple[int, int]:
         return self.own_lo - self.loc_lo, self.own_hi - self.loc_lo
 
-
-def partition(N0: int, nranks: int, rank: int, ghost: int) -> Slab:
-    """Owned ranges split as evenly as possible; ghosts clipped at the global boundary."""
-    base, extra = divmod(N0, nranks)
-    lo = rank * base + min(rank, extra)
-    hi = lo + base + (1 if rank < extra else 0)
-    if hi - lo < ghost:
-        raise ValueError(f"slab of {hi - lo} planes is thinner than the ghost width {ghost}")
-    return Slab(rank, nranks, N0, lo, hi, max(0, lo - ghost), min(N0, hi + ghost), ghost)
+    def blocks(self, T: int) -> List[int]:
+        D = self.time_block
+        return [min(D, T - t) for t in range(0, T, D)]
 
 
-def exchange_halos(local: torch.Tensor, slab: Slab, group=None) -> None:
-    """Refresh the ghost planes of `local` (leading dim = planes) from the neighbours:
-    send my first / last G owned planes down / up, receive their owned planes into my
-    ghosts.  One batch of point-to-point ops (NCCL group send/recv on GPUs)."""
-    G = slab.ghost
-    lo, hi = slab.own_local
+def _tile(h=0, w0=0, w=(0, 0, 0), hex_dim=-1, executor="auto") -> Tile:
+    return Tile(int(h), int(w0), (ctypes.c_int32 * 3)(*list(w)[:3]), int(hex_dim), EXEC[executor])
+
+
+def _desc(kind: str, ext: Sequence[int], dtype="float32"):
+    if kind not in KINDS:
+        raise StencilError(1, f"unknown stencil kind {kind!r}")
+    e = (ctypes.c_int64 * len(ext))(*[int(x) for x in ext])
+    h = ctypes.c_void_p()
+    check(lib().stencil_desc_create(ctypes.byref(h), len(ext), e, KINDS[kind], 1, None, 0, None, 0,
+                                    _dtype_code(dtype)))
+    return h
+
+
+def _layout_of(info: DistInfo, dims: int, global_ext: Sequence[int]) -> Layout:
+    return Layout(info.rank, info.nranks, tuple(int(x) for x in global_ext),
+                  tuple(int(info.local_ext[q]) for q in range(dims)), info.own_lo, info.own_hi, info.loc_lo,
+                  info.loc_hi, info.ghost, info.time_block, info.n_blocks, info.h, info.ghost_fraction)
+
+
+def layout(kind: str, global_ext: Sequence[int], T: int, rank: int, nranks: int, dtype="float32",
+           **tile) -> Layout:
+    """This rank's slab layout, exactly as stencil_plan_dist builds it (host only)."""
+    d = _desc(kind, global_ext, dtype)
+    try:
+        info = DistInfo()
+        t = _tile(**tile)
+        check(lib().stencil_dist_layout(d, int(T), ctypes.byref(t), int(rank), int(nranks), 0, ctypes.byref(info)))
+        return _layout_of(info, len(global_ext), global_ext)
+    finally:
+        lib().stencil_destroy(d)
+
+
+def exchange_halos(local: torch.Tensor, lay: Layout, group=None) -> None:
+    """The library's halo step over torch.distributed (for CPU/gloo tests of the protocol):
+    send my first / last G owned planes down / up, receive the neighbours' into my ghosts."""
+    G = lay.ghost
+    lo, hi = lay.own_local
     ops = []
-    if slab.rank > 0:
-        ops.append(dist.P2POp(dist.isend, local[lo:lo + G], slab.rank - 1, group))
-        ops.append(dist.P2POp(dist.irecv, local[lo - G:lo], slab.rank - 1, group))
-    if slab.rank < slab.nranks - 1:
-        ops.append(dist.P2POp(dist.isend, local[hi - G:hi], slab.rank + 1, group))
-        ops.append(dist.P2POp(dist.irecv, local[hi:hi + G], slab.rank + 1, group))
+    if lay.rank > 0:
+        ops.append(dist.P2POp(dist.isend, local[lo:lo + G].contiguous(), lay.rank - 1, group))
+        ops.append(dist.P2POp(dist.irecv, local[lo - G:lo], lay.rank - 1, group))
+    if lay.rank < lay.nranks - 1:
+        ops.append(dist.P2POp(dist.isend, local[hi - G:hi].contiguous(), lay.rank + 1, group))
+        ops.append(dist.P2POp(dist.irecv, local[hi:hi + G], lay.rank + 1, group))
     if ops:
         for req in dist.batch_isend_irecv(ops):
             req.wait()
 
 
-def time_blocks(T: int, D: int) -> List[int]:
-    """Block lengths: D steps each, the remainder last."""
-    out = [D] * (T // D)
-    if T % D:
-        out.append(T % D)
-    return out
+def run_protocol(local: torch.Tensor, lay: Layout, T: int, compute: Callable[[torch.Tensor, int], None],
+                 group=None) -> torch.Tensor:
+    """The distributed run of csrc/dist.cpp::run_dist with an injected per-block compute and a
+    torch.distributed exchange: for each block, exchange (but before the first), then D steps."""
+    for k, steps in enumerate(lay.blocks(T)):
+        if k > 0 and lay.nranks > 1:
+            exchange_halos(local, lay, group)
+        compute(local, steps)
+    return local
 
 
-class SlabRunner:
-    """Runs `T` steps of a stencil on a slab-partitioned grid.
+class DistPlan:
+    """A distributed plan (stencil_plan_dist) of T steps of `kind` on the global grid
+    `global_ext`, over the ranks of `group` (one GPU each).  Collective constructor."""
 
-    compute(local_tensor, steps) advances the local grid by `steps` steps in place; by
-    default it is the C-ABI hybrid-tiled path on the rank's GPU (one Plan per distinct
-    block length, built once)."""
-
-    def __init__(self, kind: str, global_extents: Sequence[int], T: int, D: int = 64,
-                 group=None, compute: Optional[Callable[[torch.Tensor, int], None]] = None,
-                 dtype=torch.float32, **tile):
+    def __init__(self, kind: str, global_ext: Sequence[int], T: int, group=None, dtype="float32", **tile):
         self.kind = kind
-        self.ext = tuple(int(e) for e in global_extents)
+        self.global_ext = tuple(int(e) for e in global_ext)
         self.T = int(T)
-        self.D = int(max(1, min(D, T))) if T > 0 else 1
         self.group = group
-        self.rank = dist.get_rank(group)
-        self.nranks = dist.get_world_size(group)
-        self.slab = partition(self.ext[0], self.nranks, self.rank, ghost=self.D)
-        self.local_ext = (self.slab.local_extent,) + self.ext[1:]
-        self.blocks = time_blocks(self.T, self.D)
-        self._compute = compute
-        self._plans = {}
-        self._tile = tile
-        self._dtype = dtype
+        self.rank = dist.get_rank(group) if dist.is_initialized() else 0
+        self.nranks = dist.get_world_size(group) if dist.is_initialized() else 1
+        emu = os.environ.get("HEXS_DIST_EMULATE_RANK")  # "r/P": play rank r of P alone (projection)
+        if emu:
+            r, P = (int(x) for x in emu.split("/"))
+            os.environ["HEXS_DIST_EMULATE"] = "1"
+            self.rank, self.nranks = r, P
+        self._d = _desc(kind, self.global_ext, dtype)
+        uid = (ctypes.c_char * 128)()
+        if self.rank == 0:
+            check(lib().stencil_dist_unique_id(uid))
+        if self.nranks > 1 and not emu:
+            obj = [bytes(uid) if self.rank == 0 else None]
+            dist.broadcast_object_list(obj, src=dist.get_global_rank(group, 0) if group is not None else 0,
+                                       group=group)
+            ctypes.memmove(uid, obj[0], 128)
+        t = _tile(**tile)
+        h = ctypes.c_void_p()
+        check(lib().stencil_plan_dist(ctypes.byref(h), self._d, self.T, ctypes.byref(t), uid, self.rank,
+                                      self.nranks, 0))
+        self._h = h
+        info = DistInfo()
+        check(lib().stencil_dist_info(h, ctypes.byref(info)))
+        self.layout = _layout_of(info, len(self.global_ext), self.global_ext)
+        self.launches_per_run = int(info.launches_per_run)
+        self._ws = None
+        self.dtype = dtype
 
-    def _gpu_compute(self, local: torch.Tensor, steps: int) -> None:
-        from .api import Plan, Stencil
+    # ---- data placement ---------------------------------------------------------------
+    def scatter(self, global_grid) -> torch.Tensor:
+        """This rank's local slab (owned + ghost planes) of a full global grid, on its GPU."""
+        lay = self.layout
+        part = global_grid[lay.loc_lo:lay.loc_hi]
+        t = part if isinstance(part, torch.Tensor) else torch.from_numpy(part.copy())
+        return t.contiguous().cuda()
 
-        plan = self._plans.get(steps)
-        if plan is None:
-            st = Stencil(self.kind, self.local_ext, dtype=self._dtype)
-            plan = self._plans[steps] = Plan(st, steps, **self._tile)
-        plan.run(local, out=local)
+    def owned(self, local: torch.Tensor) -> torch.Tensor:
+        lo, hi = self.layout.own_local
+        return local[lo:hi]
 
-    def compute(self, local: torch.Tensor, steps: int) -> None:
-        if self._compute is not None:
-            self._compute(local, steps)
-        else:
-            self._gpu_compute(local, steps)
+    # ---- execution ----------------------------------------------------------------------
+    @property
+    def block_plan(self):
+        """Borrowed handle of the D-step local plan (introspection / per-launch profiling)."""
+        bp = ctypes.c_void_p()
+        check(lib().stencil_dist_block_plan(self._h, 0, ctypes.byref(bp)))
+        return bp
 
-    def scatter_view(self, global_grid) -> torch.Tensor:
-        """The rank's local part (owned + ghost planes) of a full global grid."""
-        s = self.slab
-        return global_grid[s.loc_lo:s.loc_hi]
+    def _ensure_workspace(self, device):
+        n = ctypes.c_size_t()
+        check(lib().stencil_plan_workspace_size(self._h, ctypes.byref(n)))
+        if n.value == 0:
+            return
+        if self._ws is None or self._ws.device != device:
+            self._ws = torch.empty(n.value + 256, dtype=torch.uint8, device=device)
+        ptr = (self._ws.data_ptr() + 255) // 256 * 256
+        check(lib().stencil_plan_set_workspace(self._h, ctypes.c_void_p(ptr), n.value))
 
-    def run(self, local: torch.Tensor) -> torch.Tensor:
-        """Advance `local` (owned + ghost planes, ghosts valid at level 0) by T steps.
-        Returns local; its owned planes hold level T."""
-        for i, steps in enumerate(self.blocks):
-            if i > 0:
-                exchange_halos(local, self.slab, self.group)
-            self.compute(local, steps)
-        return local
+    def run(self, local: torch.Tensor, out: Optional[torch.Tensor] = None, stream=None) -> torch.Tensor:
+        """Collective: T steps; `local` holds level 0 on every plane of the slab.  Returns the
+        slab whose owned planes hold level T (in place unless `out` is given)."""
+        lay = self.layout
+        if not local.is_cuda or not local.is_contiguous() or tuple(local.shape) != lay.local_ext:
+            raise StencilError(1, f"local slab must be a contiguous CUDA tensor of shape {lay.local_ext}")
+        if out is None:
+            out = local
+        elif tuple(out.shape) != lay.local_ext or not out.is_contiguous() or out.device != local.device:
+            raise StencilError(1, "out must match the local slab")
+        self._ensure_workspace(local.device)
+        if stream is None:
+            stream = torch.cuda.current_stream(local.device)
+        ip = (ctypes.c_void_p * 1)(local.data_ptr())
+        op = (ctypes.c_void_p * 1)(out.data_ptr())
+        check(lib().stencil_run(self._h, ip, op, self.T, ctypes.c_void_p(stream.cuda_stream)))
+        return out
 
     def updates(self) -> int:
         """Interior points x T of the GLOBAL problem (the metric's numerator)."""
         n = 1
-        for e in self.ext:
+        for e in self.global_ext:
             n *= e - 2
         return n * self.T
 
-    def redundant_fraction(self) -> float:
-        s = self.slab
-        return (s.local_extent - (s.own_hi - s.own_lo)) / max(1, s.own_hi - s.own_lo)
+    def __del__(self):
+        if _lib._lib is None:
+            return
+        for attr in ("_h", "_d"):
+            h = getattr(self, attr, None)
+            if h is not None and h.value:
+                _lib._lib.stencil_destroy(h)
+                setattr(self, attr, None)
 
 
-def bench_main(args, cfg, configs, metric, helpers=None):
-    """bench.py --gpus N under torchrun: weak scaling, each rank owns the config's grid.
-    `helpers` is the bench module (clock sampler, roofline model, peaks)."""
+def bench_main(args, cfg, configs, metric, helpers):
+    """bench.py under torchrun (or HEXS_FORCE_DIST=1 at N = 1): every rank runs its slab of the
+    config's grid through a distributed plan.  Weak scaling for the configs whose outer extent
+    grows with N (`weak`), strong scaling for the fixed-size 3D grid."""
     import stencil_inputs
 
-    kind, ext, T, cname = configs[cfg]
-    rank = int(os.environ["RANK"])
-    world = int(os.environ["WORLD_SIZE"])
+    kind, ext, T, cname = configs[cfg][:4]
+    scaling = configs[cfg][4] if len(configs[cfg]) > 4 else "weak"
+    rank = int(os.environ.get("RANK", "0"))
+    world = int(os.environ.get("WORLD_SIZE", "1"))
     local_rank = int(os.environ.get("LOCAL_RANK", "0"))
     torch.cuda.set_device(local_rank)
-    dist.init_process_group("nccl", device_id=torch.device("cuda", local_rank))
-    gext = (ext[0] * world,) + tuple(ext[1:])
-    D = int(os.environ.get("HEXS_TIME_BLOCK", "128"))
-    runner = SlabRunner(kind, gext, T, D=D)
+    if "RANK" not in os.environ:  # a single process (N = 1 without torchrun): a group of one
+        import socket
 
-    # each rank generates only its local planes of the global synthetic grid (same recipe)
-    s = runner.slab
+        sk = socket.socket()
+        sk.bind(("127.0.0.1", 0))
+        os.environ.update({"RANK": "0", "WORLD_SIZE": "1", "LOCAL_RANK": "0", "MASTER_ADDR": "127.0.0.1",
+                           "MASTER_PORT": str(sk.getsockname()[1])})
+        sk.close()
+    if not dist.is_initialized():
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local_rank))
+    gext = ((ext[0] * world,) + tuple(ext[1:])) if scaling == "weak" else tuple(ext)
+    dp = DistPlan(kind, gext, T)
+    lay = dp.layout
     plane = 1
     for e in gext[1:]:
         plane *= e
-    local_np = stencil_inputs.uniform((s.local_extent,) + tuple(gext[1:]), seed=0, offset=s.loc_lo * plane)
+    # each rank generates only its slab of the global synthetic grid (same counter-based recipe)
+    local_np = stencil_inputs.uniform(lay.local_ext, seed=0, offset=lay.loc_lo * plane)
     host_in = torch.from_numpy(local_np).pin_memory()
     local0 = host_in.cuda()
     local = torch.empty_like(local0)
     stream = torch.cuda.current_stream()
 
     def step():
-        local.copy_(local0)
-        runner.run(local)
+        dp.run(local0, local)
 
     for _ in range(max(3, args.warmup)):
         step()
     torch.cuda.synchronize()
     dist.barrier()
     e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-    sampler = helpers.ClockSampler(local_rank) if helpers is not None else None
-    if sampler is not None:
-        sampler.__enter__()
+    sampler = helpers.ClockSampler(local_rank)
+    sampler.__enter__()
+    torch.cuda.synchronize()
+    dist.barrier()
     e0.record(stream)
     for _ in range(args.steps):
         step()
     e1.record(stream)
     torch.cuda.synchronize()
-    if sampler is not None:
-        sampler.__exit__(None, None, None)
+    sampler.__exit__(None, None, None)
     ms = torch.tensor([e0.elapsed_time(e1) / args.steps], device="cuda")
     dist.all_reduce(ms, op=dist.ReduceOp.MAX)
     ms = float(ms.item())
-    value = runner.updates() / (ms * 1e-3) / 1e9
+    value = dp.updates() / (ms * 1e-3) / 1e9
 
-    # end to end through the public API: pinned H2D of the rank's slab, the run (halo
-    # exchanges included), D2H of the owned planes; two slab buffers and H2D / D2H streams
-    # overlap a step's transfers with its neighbours' compute (as the single-GPU bench does)
-    lo, hi = s.own_local
+    # end to end through the public API: pinned H2D of the rank's slab, the distributed run
+    # (halo exchanges included), D2H of the owned planes; two slab buffer pairs and H2D / D2H
+    # streams overlap a step's transfers with its neighbours' compute
+    lo, hi = lay.own_local
     host_out = [torch.empty_like(host_in[lo:hi]).pin_memory() for _ in range(2)]
-    locs = [local, torch.empty_like(local)]
+    ins = [local0, torch.empty_like(local0)]
+    outs = [local, torch.empty_like(local)]
     h2d, d2h = torch.cuda.Stream(), torch.cuda.Stream()
     ev_in = [torch.cuda.Event() for _ in range(2)]
     ev_done = [torch.cuda.Event() for _ in range(2)]
     ev_out = [torch.cuda.Event() for _ in range(2)]
-    for k in range(2):  # warm both slab buffers (the library captures a CUDA graph per pointer set)
-        for _ in range(2):
-            locs[k].copy_(local0)
-            runner.run(locs[k])
-    dist.barrier()
+    for k in range(2):
+        ins[k].copy_(local0)
+        dp.run(ins[k], outs[k])
     torch.cuda.synchronize()
+    dist.barrier()
     f0, f1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
     f0.record(stream)
     h2d.wait_event(f0)
@@ -220,20 +301,17 @@ def bench_main(args, cfg, configs, metric, helpers=None):
         k = i % 2
         with torch.cuda.stream(h2d):
             if i >= 2:
-                # the slab buffer is both input and output: its previous step's compute AND
-                # the download of that step's result must be done before it is overwritten
-                h2d.wait_event(ev_done[k])
-                h2d.wait_event(ev_out[k])
-            locs[k].copy_(host_in, non_blocking=True)
+                h2d.wait_event(ev_done[k])  # step i-2 consumed this input slab
+            ins[k].copy_(host_in, non_blocking=True)
             ev_in[k].record(h2d)
         stream.wait_event(ev_in[k])
         if i >= 2:
-            stream.wait_event(ev_out[k])
-        runner.run(locs[k])
+            stream.wait_event(ev_out[k])  # step i-2's result has left this output slab
+        dp.run(ins[k], outs[k])
         ev_done[k].record(stream)
         with torch.cuda.stream(d2h):
             d2h.wait_event(ev_done[k])
-            host_out[k].copy_(locs[k][lo:hi], non_blocking=True)
+            host_out[k].copy_(outs[k][lo:hi], non_blocking=True)
             ev_out[k].record(d2h)
     stream.wait_event(ev_out[(args.steps - 1) % 2])
     stream.wait_event(ev_out[args.steps % 2])
@@ -242,50 +320,59 @@ def bench_main(args, cfg, configs, metric, helpers=None):
     e2e_ms = torch.tensor([f0.elapsed_time(f1) / args.steps], device="cuda")
     dist.all_reduce(e2e_ms, op=dist.ReduceOp.MAX)
     e2e_ms = float(e2e_ms.item())
-    # the pipelined result equals a device-resident run's owned planes
-    ref = local0.clone()
-    runner.run(ref)
-    torch.cuda.synchronize()
-    assert torch.equal(host_out[(args.steps - 1) % 2], ref[lo:hi].cpu()), "pipelined e2e result differs"
-    host_out = host_out[0]
+    # the pipelined result equals the device-resident run's owned planes
+    assert torch.equal(host_out[(args.steps - 1) % 2], local[lo:hi].cpu()), "pipelined e2e result differs"
 
-    # phase-kernel roofline of the main block plan (algorithmic bytes / measured launch time)
+    # phase-kernel roofline of the D-step block plan: kernel-region events of one run
+    bp = dp.block_plan
+    check(lib().stencil_plan_profile(bp, 1))
+    dp.run(local0, local)
+    kms, nl, mx = ctypes.c_double(), ctypes.c_int64(), ctypes.c_double()
+    check(lib().stencil_plan_profile_read(bp, ctypes.byref(kms), ctypes.byref(nl), ctypes.byref(mx)))
+    check(lib().stencil_plan_profile(bp, 0))
+    binfo = _lib.PlanInfo()
+    check(lib().stencil_plan_info(bp, ctypes.byref(binfo)))
+    bpu = 4 * (binfo.tile_in + binfo.tile_out) / binfo.tile_points
+    upd_block = binfo.updates  # one D-step block on the local slab (ghost planes included)
+    peak, peak_src = helpers.load_peaks()
     roof = None
-    plan = runner._plans.get(runner.D)
-    launches = sum(runner._plans[b].info["n_launches"] for b in runner.blocks)
-    if plan is not None and helpers is not None:
-        plan.profile(1)
-        step()
-        prof = plan.profile_read()
-        plan.profile(0)
-        info = plan.info
-        bpu = helpers.bytes_per_update_tiled(info, 4, plan)
-        avg = prof["kernel_ms"] / max(1, prof["launches"])
-        alg = info["updates"] / info["n_launches"] * bpu
-        peak, peak_src = helpers.load_peaks()
-        roof = {"bound": "hbm", "achieved": alg / (avg * 1e-3) / 1e9, "peak": peak, "unit": "GB/s",
-                "frac": alg / (avg * 1e-3) / 1e9 / peak, "traffic": None, "peak_source": peak_src,
-                "kernel": helpers.KERNEL_NAMES.get(plan.executor_name, plan.executor_name),
-                "bytes_per_update": bpu, "avg_launch_ms": avg}
+    if nl.value > 0:
+        achieved = upd_block * bpu / (kms.value * 1e-3) / 1e9
+        roof = {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s", "frac": achieved / peak,
+                "traffic": None, "peak_source": peak_src,
+                "kernel": helpers.KERNEL_NAMES.get(_lib.KERNELS[binfo.kernel], _lib.KERNELS[binfo.kernel]),
+                "bytes_per_update": bpu, "block_kernel_ms": kms.value, "block_launches": nl.value,
+                "note": "one D-step block plan on the local slab (ghost planes included); block-cut "
+                        "and ghost traffic not in bytes_per_update"}
     if rank == 0:
         nbytes_in = host_in.numel() * host_in.element_size()
-        nbytes_out = host_out.numel() * host_out.element_size()
+        nbytes_out = host_out[0].numel() * host_out[0].element_size()
         line = {"metric": metric, "value": value, "unit": "GStencil-updates/s", "n_gpus": world,
                 "steps": args.steps, "warmup": args.warmup, "ms_per_step": ms,
-                "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "f32",
+                "higher_is_better": True, "scaling": scaling, "vs_baseline": None, "dtype": "f32",
                 "data": "synthetic",
-                "config": {"workload": cname + f" weak-scaled to {gext[0]} planes over {world} GPUs",
-                           "kind": kind, "extents": list(gext), "T": T, "time_block": runner.D,
-                           "ghost_planes": runner.slab.ghost,
-                           "redundant_fraction": runner.redundant_fraction(),
+                "config": {"workload": cname + (f" weak-scaled to {gext[0]} planes over {world} GPUs"
+                                                if scaling == "weak" else f" over {world} GPUs"),
+                           "kind": kind, "extents": list(gext), "T": T, "partition": "dim 0 slabs",
+                           "time_block": lay.time_block, "ghost_planes": lay.ghost,
+                           "ghost_fraction": lay.ghost_fraction, "local_extents": list(lay.local_ext),
                            "l2": "inputs larger than L2 (per-rank slab > 126 MB)"},
                 "roofline": roof,
                 "cpu_baseline": None,
-                "e2e": {"value": runner.updates() / (e2e_ms * 1e-3) / 1e9, "unit": "GStencil-updates/s",
+                "e2e": {"value": dp.updates() / (e2e_ms * 1e-3) / 1e9, "unit": "GStencil-updates/s",
                         "h2d_bytes_per_step": nbytes_in * world, "d2h_bytes_per_step": nbytes_out * world,
                         "ms_per_step": e2e_ms,
-                        "pipelined": "2 slab buffers; H2D and D2H streams overlap the neighbouring steps' compute"},
-                "gpu_launches": launches * args.steps,
-                "clocks": sampler.summary() if sampler is not None else None}
+                        "pipelined": "2 slab buffer pairs; H2D and D2H streams overlap the neighbouring steps' compute"},
+                "gpu_launches": dp.launches_per_run * args.steps,
+                "clocks": sampler.summary()}
+        emu = os.environ.get("HEXS_DIST_EMULATE_RANK")
+        if emu:  # a projection, not a measurement of N GPUs: say so and report the rank's rate
+            r, P = (int(x) for x in emu.split("/"))
+            own = lay.own_hi - lay.own_lo
+            line["emulated_rank"] = {"rank": r, "nranks": P, "owned_planes": own,
+                                     "rank_gups": value * own / gext[0],
+                                     "note": "one GPU runs rank r's slab alone (ghosts fixed, no NCCL): compute-only "
+                                             "projection; 'value' is the whole-grid rate of that rank's time"}
         print(json.dumps(line), flush=True)
+    dist.barrier()
     dist.destroy_process_group()

@@ -187,35 +187,32 @@ def test_full_size_fdtd():
         assert_bitexact(a, b, f"fdtd 8192^2 T=500 {name}")
 
 
-def test_slab_runner_nccl_single_rank():
-    """The multi-GPU slab path (paper_conf_cgo_grosserchsv14_b200/dist.py) on the GPU with a
-    one-rank NCCL process group: time blocks of D steps run back to back through the C-ABI
-    plans (including a remainder block) must reproduce the single-domain oracle bit-exactly."""
+def test_dist_plan_nccl_single_rank():
+    """The C ABI's distributed plan (stencil_plan_dist: NCCL communicator from a unique id,
+    time blocks of D steps, block plans on the local slab) with one rank on the GPU: bit-exact
+    against the single-domain oracle, including a remainder block and both dtypes' 2D/3D paths."""
     import os
-    import socket
-
-    import torch.distributed as tdist
 
     from paper_conf_cgo_grosserchsv14_b200 import dist as hdist
 
-    sock = socket.socket()
-    sock.bind(("127.0.0.1", 0))
-    port = sock.getsockname()[1]
-    sock.close()
-    store = tdist.TCPStore("127.0.0.1", port, 1, True)
-    tdist.init_process_group("nccl", store=store, rank=0, world_size=1,
-                             device_id=torch.device("cuda", 0))
-    try:
-        for kind, ext, T, D in [("star2d5", (301, 517), 37, 16), ("star3d7", (40, 45, 68), 11, 4)]:
+    for kind, ext, T, D in [("star2d5", (301, 517), 37, "16"), ("star3d7", (40, 45, 68), 11, "4"),
+                            ("star3d7", (64, 40, 64), 20, ""), ("box2d9", (130, 260), 19, "")]:
+        if D:
+            os.environ["HEXS_TIME_BLOCK"] = D
+        else:
+            os.environ.pop("HEXS_TIME_BLOCK", None)
+        try:
             g = stencil_inputs.uniform(ext, seed=9)
-            runner = hdist.SlabRunner(kind, ext, T, D=D)
-            local = torch.from_numpy(np.ascontiguousarray(runner.scatter_view(g))).cuda()
-            runner.run(local)
+            dp = hdist.DistPlan(kind, ext, T)
+            assert dp.layout.loc_lo == 0 and dp.layout.loc_hi == ext[0]
+            local = dp.scatter(g)
+            out = torch.empty_like(local)
+            for _ in range(2):
+                dp.run(local, out)
             torch.cuda.synchronize()
-            assert_bitexact(local.cpu().numpy(), oracle.run(kind, g, T), f"slab {kind} D={D}")
-    finally:
-        tdist.destroy_process_group()
-
+            assert_bitexact(dp.owned(out).cpu().numpy(), oracle.run(kind, g, T), f"dist {kind} D={D}")
+        finally:
+            os.environ.pop("HEXS_TIME_BLOCK", None)
 
 @pytest.mark.parametrize("kind,shape,T", [("star2d5", (300, 1030), 19), ("box2d9", (257, 1100), 12),
                                           ("star3d7", (40, 45, 68), 11), ("box3d27", (30, 37, 68), 9)])
