@@ -72,6 +72,10 @@ def lib() -> ctypes.CDLL:
             p.argtypes = [ctypes.c_int, ctypes.c_int, i64p, dp, ctypes.c_int, ctypes.c_int64,
                           ctypes.c_void_p, ctypes.c_int, i64p, ctypes.c_void_p]
             p.restype = ctypes.c_int
+            li = getattr(L, f"oracle_linear_{T}")
+            li.argtypes = [ctypes.c_int, i64p, ctypes.c_int, ctypes.POINTER(ctypes.c_int), dp, ctypes.c_int64,
+                           ctypes.c_void_p, ctypes.c_void_p, ctypes.c_int]
+            li.restype = ctypes.c_int
         L.oracle_max_threads.restype = ctypes.c_int
         _lib = L
     return _lib
@@ -140,3 +144,21 @@ def points(kind: str, grid: np.ndarray, steps: int, coords: np.ndarray,
     if rc != 0:
         raise ValueError(f"oracle_points failed rc={rc}")
     return vals
+
+
+def linear(grid: np.ndarray, offsets: Sequence[Sequence[int]], coefficients: Sequence[float], steps: int,
+           nthreads: int = 1) -> np.ndarray:
+    """General linear stencil (oracle.c `oracle_linear`): level `steps` of
+    A'[p] = c_0 A[p+o_0] + ... + c_{n-1} A[p+o_{n-1}] (left to right) over the interior
+    [R, N-1-R], R = max |offset|."""
+    a = np.ascontiguousarray(grid)
+    offs = np.ascontiguousarray(np.asarray(offsets, dtype=np.int32).reshape(-1, a.ndim))
+    coefs = [float(c) for c in coefficients]
+    assert offs.shape[0] == len(coefs)
+    out = np.empty_like(a)
+    f = getattr(lib(), f"oracle_linear_{_ctype(a.dtype)}")
+    rc = f(a.ndim, _i64(a.shape), len(coefs), offs.ctypes.data_as(ctypes.POINTER(ctypes.c_int)), _dbl(coefs),
+           int(steps), a.ctypes.data, out.ctypes.data, int(nthreads))
+    if rc != 0:
+        raise ValueError(f"oracle_linear failed rc={rc}")
+    return out

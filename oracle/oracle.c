@@ -290,6 +290,64 @@ ORACLE_FDTD(double)
 ORACLE_POINTS(float)
 ORACLE_POINTS(double)
 
+/* ------------------------------------------------------------------------------------
+ * General linear stencil ("general descriptors"): any access set
+ * of n offsets o_k (2D or 3D, any radius) with coefficients c_k, evaluated left to right
+ *     acc = c_0 * A[p + o_0];  acc = acc + c_k * A[p + o_k]  (k = 1 .. n-1)
+ * over the interior [R, N_d-1-R] of every dimension, R = max |o_k,d| (the cells within R of
+ * an edge are Dirichlet, never written); the same ping-pong time loop as oracle_run (Fig. 1,
+ * PAPER.md:142-148).  offs: n*dims int32 (slow -> fast), coefs: n doubles rounded once to T.
+ * ---------------------------------------------------------------------------------- */
+#define ORACLE_LINEAR(T)                                                               \
+  int oracle_linear_##T(int dims, const int64_t *ext, int n, const int *offs,          \
+                        const double *coefs, int64_t steps, const T *in, T *out,       \
+                        int nthreads) {                                                \
+    if ((dims != 2 && dims != 3) || n < 1 || n > 125 || steps < 0) return 1;           \
+    int64_t N[3] = {ext[0], ext[1], dims == 3 ? ext[2] : 1};                           \
+    int64_t st[3] = {dims == 3 ? N[1] * N[2] : N[1], dims == 3 ? N[2] : 1, 1};         \
+    int R = 0;                                                                         \
+    int64_t delta[125];                                                                \
+    T c[125];                                                                          \
+    for (int k = 0; k < n; ++k) {                                                      \
+      delta[k] = 0;                                                                    \
+      for (int d = 0; d < dims; ++d) {                                                 \
+        int o = offs[k * dims + d];                                                    \
+        if (o > R) R = o;                                                              \
+        if (-o > R) R = -o;                                                            \
+        delta[k] += (int64_t)o * st[d];                                                \
+      }                                                                                \
+      c[k] = (T)coefs[k];                                                              \
+    }                                                                                  \
+    if (dims == 2) N[2] = 1 + 2 * (int64_t)R; /* the loop below runs x in [R, N2-1-R] */ \
+    int64_t n_el = N[0] * N[1] * (dims == 3 ? N[2] : 1);                               \
+    T *buf[2];                                                                         \
+    buf[0] = out;                                                                      \
+    buf[1] = (T *)malloc((size_t)n_el * sizeof(T));                                    \
+    if (!buf[1]) return 2;                                                             \
+    memmove(buf[0], in, (size_t)n_el * sizeof(T));                                     \
+    memcpy(buf[1], in, (size_t)n_el * sizeof(T));                                      \
+    if (nthreads < 1) nthreads = 1;                                                    \
+    for (int64_t t = 0; t < steps; ++t) {                                              \
+      const T *src = buf[t % 2];                                                       \
+      T *dst = buf[(t + 1) % 2];                                                       \
+      _Pragma("omp parallel for schedule(static) num_threads(nthreads)")               \
+      for (int64_t a = R; a < N[0] - R; ++a)                                           \
+        for (int64_t b = R; b < N[1] - R; ++b)                                         \
+          for (int64_t x = R; x < N[2] - R; ++x) {                                     \
+            int64_t p = dims == 3 ? a * st[0] + b * st[1] + x : a * st[0] + b;         \
+            T acc = c[0] * src[p + delta[0]];                                          \
+            for (int k = 1; k < n; ++k) acc = acc + c[k] * src[p + delta[k]];          \
+            dst[p] = acc;                                                              \
+          }                                                                            \
+    }                                                                                  \
+    if (steps % 2 == 1) memcpy(out, buf[1], (size_t)n_el * sizeof(T));                 \
+    free(buf[1]);                                                                      \
+    return 0;                                                                          \
+  }
+
+ORACLE_LINEAR(float)
+ORACLE_LINEAR(double)
+
 /* Threads the OpenMP runtime would use (reported as `cores` by bench.py). */
 int oracle_max_threads(void) {
 #ifdef _OPENMP
