@@ -56,7 +56,10 @@ typedef enum {
   STENCIL_STAR3D7 = 4,     /* laplacian/heat 3D 7-pt: c0*c + c1*(((((n+s)+w)+e)+u)+d)     */
   STENCIL_GRADIENT3D = 5,  /* c + 1/sqrt(eps + sum_6 (c-nb)^2)   (eps = 1e-2)             */
   STENCIL_BOX3D27 = 6,     /* heat 3D 27-pt: k * lexicographic sum of the 3x3x3 box (1/27)*/
-  STENCIL_GRADIENT2D = 7   /* c + 1/sqrt(eps + sum_4 (c-nb)^2)   (eps = 1e-2)             */
+  STENCIL_GRADIENT2D = 7,  /* c + 1/sqrt(eps + sum_4 (c-nb)^2)   (eps = 1e-2)             */
+  STENCIL_LINEAR = 8       /* general linear stencil, 2D or 3D, any access set and radius:
+                              c_0*A[p+o_0] + c_1*A[p+o_1] + ... (left to right); offsets and
+                              coefficients required (n <= 64); radius = max |o| */
 } stencil_kind;
 
 typedef struct stencil_desc_s *stencil_desc_t;
@@ -87,11 +90,13 @@ enum {
  *   dims        2 or 3 (must match the class)
  *   extents     dims values, slow -> fast, each >= 3 (boundary included)
  *   kind        stencil class
- *   radius      1 (every implemented class has radius 1)
+ *   radius      1 for the fixed classes; STENCIL_LINEAR: max |offset| over its access set
  *   offsets     optional (may be NULL): n_offsets*dims int32 offsets; if given they must
- *               equal the class's access set (validated, order free)
+ *               equal the class's access set (validated, order free).  STENCIL_LINEAR:
+ *               required, 1..64 offsets, evaluated in the given order
  *   coefficients optional (NULL = class defaults): n_coefficients doubles, rounded once
- *               to the working precision (see stencil_kind for the count and meaning)
+ *               to the working precision (see stencil_kind for the count and meaning);
+ *               STENCIL_LINEAR: required, one per offset
  *   dtype       STENCIL_F32 or STENCIL_F64 (the arithmetic precision)
  * Host only; does not touch the GPU. */
 stencil_status stencil_desc_create(stencil_desc_t *out, int dims, const int64_t *extents,
@@ -272,6 +277,23 @@ stencil_status stencil_plan_schedule_of(stencil_plan_t plan, int64_t tau, const 
 stencil_status stencil_plan_profile(stencil_plan_t plan, int max_runs);
 stencil_status stencil_plan_profile_read(stencil_plan_t plan, double *kernel_ms, int64_t *launches,
                                          double *max_launch_ms);
+
+/* The tile-size model (a2; Sec. 3.7): for a hexagon (h, w0) along hex_dim,
+ * the exact per-column points / In / Out of the full hexagon, the load-to-compute ratio as HBM
+ * bytes per update, and the two B200 terms -- the unrolled body against the instruction cache
+ * (family 1 = 2D register-wavefront kernel, 2 = 3D tile-wavefront kernel, 0 = generic kernel:
+ * no code term) and the CTA-count (wave) efficiency -- with the predicted relative rate.
+ * `selected` = 1 if the planner's automatic choice for this family is this tile.  Host only. */
+typedef struct {
+  int32_t h, w0;
+  int64_t points, in, out;
+  double bytes_per_update, body_bytes, code_eff;
+  int64_t ctas, slots;
+  double wave_eff, rate;
+  int32_t selected;
+} stencil_tile_eval_t;
+stencil_status stencil_tile_model(stencil_desc_t desc, int h, int w0, int hex_dim, int family,
+                                  stencil_tile_eval_t *out);
 
 int stencil_abi_version(void);
 

@@ -69,7 +69,7 @@ def _units():
     headers = [os.path.join(dp, f) for dp, _, fs in os.walk(CSRC) for f in fs
                if f.endswith((".h", ".cuh"))] + [os.path.join(ROOT, "include", "stencil.h")]
     units = []
-    for src in ["desc.cpp", "plan.cpp", "dist.cpp"]:
+    for src in ["desc.cpp", "plan.cpp", "dist.cpp", "tilemodel.cpp"]:
         units.append((os.path.join(CSRC, src), "cxx", []))
     for src in ["run.cu", "kernels/generic.cu", "kernels/registry.cu", "kernels/fdtd.cu"]:
         units.append((os.path.join(CSRC, src), "nvcc", []))

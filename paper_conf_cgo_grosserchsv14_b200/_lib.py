@@ -18,7 +18,7 @@ STATUS = {0: "STENCIL_OK", 1: "STENCIL_E_INVALID", 2: "STENCIL_E_UNSUPPORTED",
           6: "STENCIL_E_NCCL"}
 
 KINDS = {"jacobi2d5": 0, "star2d5": 1, "box2d9": 2, "fdtd2d": 3, "star3d7": 4,
-         "gradient3d": 5, "box3d27": 6, "gradient2d": 7}
+         "gradient3d": 5, "box3d27": 6, "gradient2d": 7, "linear": 8}
 EXEC = {"auto": 0, "generic": 1, "naive": 2}
 
 # every symbol include/stencil.h declares
@@ -28,7 +28,7 @@ SYMBOLS = ["stencil_desc_create", "stencil_desc_deps", "stencil_plan",
            "stencil_plan_launches", "stencil_plan_hexagon", "stencil_plan_schedule_of",
            "stencil_plan_profile", "stencil_plan_profile_read", "stencil_abi_version",
            "stencil_dist_unique_id", "stencil_dist_layout", "stencil_plan_dist", "stencil_dist_info",
-           "stencil_dist_block_plan"]
+           "stencil_dist_block_plan", "stencil_tile_model"]
 
 
 class StencilError(RuntimeError):
@@ -67,6 +67,14 @@ class DistInfo(ctypes.Structure):
                 ("loc_hi", ctypes.c_int64), ("ghost", ctypes.c_int64), ("time_block", ctypes.c_int64),
                 ("n_blocks", ctypes.c_int64), ("h", ctypes.c_int32), ("ghost_fraction", ctypes.c_double),
                 ("launches_per_run", ctypes.c_int64)]
+
+
+class TileEval(ctypes.Structure):
+    _fields_ = [("h", ctypes.c_int32), ("w0", ctypes.c_int32), ("points", ctypes.c_int64),
+                ("in_", ctypes.c_int64), ("out", ctypes.c_int64), ("bytes_per_update", ctypes.c_double),
+                ("body_bytes", ctypes.c_double), ("code_eff", ctypes.c_double), ("ctas", ctypes.c_int64),
+                ("slots", ctypes.c_int64), ("wave_eff", ctypes.c_double), ("rate", ctypes.c_double),
+                ("selected", ctypes.c_int32)]
 
 
 class Launch(ctypes.Structure):
@@ -108,6 +116,7 @@ def lib() -> ctypes.CDLL:
     L.stencil_plan_dist.argtypes = [P(vp), vp, i64, P(Tile), vp, ctypes.c_int, ctypes.c_int, ctypes.c_int]
     L.stencil_dist_info.argtypes = [vp, P(DistInfo)]
     L.stencil_dist_block_plan.argtypes = [vp, ctypes.c_int, P(vp)]
+    L.stencil_tile_model.argtypes = [vp, ctypes.c_int, ctypes.c_int, ctypes.c_int, ctypes.c_int, P(TileEval)]
     for name in SYMBOLS:
         f = getattr(L, name)
         if name not in ("stencil_last_error", "stencil_abi_version"):

@@ -47,8 +47,14 @@ class Stencil:
             flat = [int(v) for o in offsets for v in o]
             off_p = (ctypes.c_int32 * len(flat))(*flat)
             noff = len(offsets)
+        radius = 1
+        if kind == "linear":  # a general access set: its radius is the largest |offset|
+            if offsets is None or coefficients is None:
+                raise StencilError(1, "a linear stencil needs offsets and coefficients")
+            radius = max(abs(int(v)) for o in offsets for v in o)
+        self.radius = radius
         h = ctypes.c_void_p()
-        check(lib().stencil_desc_create(ctypes.byref(h), self.dims, ext, KINDS[kind], 1, off_p,
+        check(lib().stencil_desc_create(ctypes.byref(h), self.dims, ext, KINDS[kind], radius, off_p,
                                         noff, coef_p, ncoef, self.dtype_code))
         self._h = h
 

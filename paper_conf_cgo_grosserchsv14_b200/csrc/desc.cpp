@@ -7,6 +7,7 @@
 // library the memory-based distance set is finite and is enumerated in closed form here
 // (the brute-force simulation in oracle/schedule.py pins it in the tests).
 #include <algorithm>
+#include <cstdlib>
 #include <cstring>
 #include <new>
 #include <set>
@@ -57,6 +58,7 @@ static int class_dims(int kind) {
     case STENCIL_JACOBI2D5: case STENCIL_STAR2D5: case STENCIL_BOX2D9:
     case STENCIL_FDTD2D: case STENCIL_GRADIENT2D: return 2;
     case STENCIL_STAR3D7: case STENCIL_GRADIENT3D: case STENCIL_BOX3D27: return 3;
+    case STENCIL_LINEAR: return -1;  // 2 or 3
     default: return 0;
   }
 }
@@ -118,7 +120,13 @@ static void build_statements(Desc& d) {
   d.pingpong = true;
   Stmt s;
   s.write = 0;
-  for (auto& o : class_offsets(d.kind)) {
+  std::vector<std::vector<int>> offs = class_offsets(d.kind);
+  if (d.kind == STENCIL_LINEAR) {
+    offs.clear();
+    for (size_t k = 0; k * d.dims < d.loff.size(); ++k)
+      offs.push_back(std::vector<int>(d.loff.begin() + k * d.dims, d.loff.begin() + (k + 1) * d.dims));
+  }
+  for (auto& o : offs) {
     Access a{0, {0, 0, 0}};
     for (int k = 0; k < d.dims; ++k) a.off[k] = o[k];
     s.reads.push_back(a);
@@ -190,9 +198,20 @@ stencil_status stencil_desc_create(stencil_desc_t* out, int dims, const int64_t*
   *out = nullptr;
   const int cd = class_dims(kind);
   if (cd == 0) return fail(STENCIL_E_INVALID, "stencil_desc_create: unknown stencil kind");
-  if (dims != cd) return fail(STENCIL_E_INVALID, "stencil_desc_create: dims does not match the class");
+  if (cd > 0 ? dims != cd : (dims != 2 && dims != 3))
+    return fail(STENCIL_E_INVALID, "stencil_desc_create: dims does not match the class");
   if (!extents) return fail(STENCIL_E_INVALID, "stencil_desc_create: extents is NULL");
-  if (radius != 1) return fail(STENCIL_E_UNSUPPORTED, "stencil_desc_create: only radius 1 classes are implemented");
+  if (kind == STENCIL_LINEAR) {
+    if (!offsets || !coefficients || n_offsets < 1 || n_offsets > 64 || n_coefficients != n_offsets)
+      return fail(STENCIL_E_INVALID, "stencil_desc_create: LINEAR needs 1..64 offsets and one coefficient each");
+    int R = 0;
+    for (int q = 0; q < n_offsets * dims; ++q) R = std::max(R, std::abs((int)offsets[q]));
+    if (radius != R)
+      return fail(STENCIL_E_INVALID, "stencil_desc_create: radius must equal max |offset| of the access set");
+    if (R < 1 || R > 8) return fail(STENCIL_E_UNSUPPORTED, "stencil_desc_create: LINEAR radius must be in [1, 8]");
+  } else if (radius != 1) {
+    return fail(STENCIL_E_UNSUPPORTED, "stencil_desc_create: the fixed classes have radius 1");
+  }
   if (dtype != STENCIL_F32 && dtype != STENCIL_F64) return fail(STENCIL_E_INVALID, "stencil_desc_create: bad dtype");
   for (int q = 0; q < dims; ++q)
     if (extents[q] < 2 * radius + 1 || extents[q] > (int64_t(1) << 31))
@@ -207,6 +226,13 @@ stencil_status stencil_desc_create(stencil_desc_t* out, int dims, const int64_t*
   int nd = 0;
   default_coefficients(kind, d->coef, &nd);
   d->ncoef = nd;
+  if (kind == STENCIL_LINEAR) {
+    d->loff.assign(offsets, offsets + (size_t)n_offsets * dims);
+    d->lcoef.assign(coefficients, coefficients + n_offsets);
+    build_statements(*d);
+    *out = reinterpret_cast<stencil_desc_t>(d);
+    return STENCIL_OK;
+  }
   if (coefficients) {
     if (n_coefficients != nd) {
       delete d;

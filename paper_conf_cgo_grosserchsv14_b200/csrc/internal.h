@@ -49,6 +49,9 @@ struct Desc {
   int nfields = 1;
   bool pingpong = true;
   std::vector<Stmt> stmts;
+  // STENCIL_LINEAR: the access set (n x dims offsets, slow -> fast) and its coefficients
+  std::vector<int> loff;
+  std::vector<double> lcoef;
   size_t elem() const { return dtype == STENCIL_F64 ? 8 : 4; }
   int64_t points() const { return ext[0] * ext[1] * (dims == 3 ? ext[2] : 1); }
 };
@@ -148,6 +151,26 @@ int fast3d_variant(int kind, int dtype, int h, int w0, int wy);
 int fast3d_tile(int variant, int* wy, int* wx);
 bool fast3d_variant_matches(int variant, int kind, int dtype, int h, int w0);
 int stream3d_variant(int kind, int dtype, int h, int w0);
+int fast2d_variant_count();
+bool fast2d_variant_info(int variant, int* kind, int* dtype, int* h, int* w0);
+int fast3d_variant_count();
+bool fast3d_variant_info(int variant, int* kind, int* dtype, int* h, int* w0);
+
+// tilemodel.cpp: the tile-size model of Sec. 3.7 (load-to-compute ratio) with the on-chip
+// (instruction cache) and CTA-count terms of the B200 kernels
+enum TileFamily { FAMILY_GENERIC = 0, FAMILY_FAST2D = 1, FAMILY_FAST3D = 2 };
+struct TileEval {
+  int h, w0;
+  int64_t points, in, out;  // per classical column of one full hexagon
+  double bytes_per_update;  // word * (In + Out) / points
+  double body_bytes;        // unrolled level bodies of the fast kernels (instruction cache)
+  double code_eff;          // min(1, capacity / body)^3
+  int64_t ctas, slots;      // CTAs of a full launch and resident slots
+  double wave_eff;          // ctas / (waves * slots)
+  double rate;              // predicted relative rate (updates / s, up to a constant)
+};
+bool tile_eval(const Desc& d, int hd, const Rat& d0, const Rat& d1, int h, int w0, int family, TileEval* out);
+bool tile_select(const Desc& d, int hd, const Rat& d0, const Rat& d1, int family, int* h, int* w0);
 int stream3d_carry_block(int variant);  // floats per (strip, step) carry block
 
 }  // namespace hexs

@@ -18,6 +18,15 @@ namespace hexs {
 
 namespace {
 
+// K_LINEAR: the descriptor's access set in its order, products then left-to-right sums (the
+// oracle's expression tree; no contraction: --fmad=false)
+template <typename T>
+__device__ __forceinline__ T linear_point(const T* __restrict__ A, int64_t p, const LinearTerms& L) {
+  T acc = (T)L.coef[0] * A[p + L.delta[0]];
+  for (int k = 1; k < L.n; ++k) acc = acc + (T)L.coef[k] * A[p + L.delta[k]];
+  return acc;
+}
+
 template <typename T, int KIND>
 __device__ __forceinline__ void generic_point(const GenericArgs& g, int64_t tau, const int64_t* c,
                                               const Coef<T>& k) {
@@ -36,6 +45,16 @@ __device__ __forceinline__ void generic_point(const GenericArgs& g, int64_t tau,
     } else {
       if (i <= N0 - 2 && j <= N1 - 2) hz[p] = fdtd_hz<T>(hz[p], ex[p + 1], ex[p], ey[p + N1], ey[p], k);
     }
+  } else if constexpr (KIND == K_LINEAR) {
+    int64_t p = 0;
+    const int R = g.lin.R;
+    for (int q = 0; q < g.dims; ++q) {
+      if (c[q] < R || c[q] > g.N[q] - 1 - R) return;  // Dirichlet cells are never written
+      p += c[q] * g.st[q];
+    }
+    const T* src = static_cast<const T*>(g.f[tau & 1]);
+    T* dst = static_cast<T*>(g.f[(tau + 1) & 1]);
+    dst[p] = linear_point<T>(src, p, g.lin);
   } else {
     int64_t p = 0;
     for (int q = 0; q < g.dims; ++q) {
@@ -253,6 +272,21 @@ __global__ void __launch_bounds__(32 * kNaiveV4Rows) naive3d_v4_kernel(const flo
   }
 }
 
+// Naive step of a general linear stencil: one thread per interior point.
+template <typename T>
+__global__ void __launch_bounds__(256) naive_linear_kernel(const T* __restrict__ src, T* __restrict__ dst,
+                                                           int64_t N0, int64_t N1, int64_t N2,
+                                                           const __grid_constant__ LinearTerms L) {
+  const int R = L.R;
+  const int64_t x = R + blockIdx.x * (int64_t)blockDim.x + threadIdx.x;
+  const int64_t y = R + (int64_t)blockIdx.y;
+  const int64_t z = N2 > 1 ? R + (int64_t)blockIdx.z : 0;
+  const int64_t X = N2 > 1 ? N2 : N1, Y = N2 > 1 ? N1 : N0;  // 2D: (y, x) = (i, j)
+  if (x > X - 1 - R || y > Y - 1 - R) return;
+  const int64_t p = N2 > 1 ? (z * N1 + y) * N2 + x : y * N1 + x;
+  dst[p] = linear_point<T>(src, p, L);
+}
+
 template <typename T>
 __global__ void __launch_bounds__(256) naive_fdtd_kernel(T* __restrict__ ex, T* __restrict__ ey,
                                                          T* __restrict__ hz, int64_t N0, int64_t N1,
@@ -300,6 +334,7 @@ cudaError_t launch_generic_t(int kind, const GenericArgs& g, int grid, cudaStrea
     break;
     HEXS_CASE(K_JACOBI2D5) HEXS_CASE(K_STAR2D5) HEXS_CASE(K_BOX2D9) HEXS_CASE(K_FDTD2D)
     HEXS_CASE(K_STAR3D7) HEXS_CASE(K_GRADIENT3D) HEXS_CASE(K_BOX3D27) HEXS_CASE(K_GRADIENT2D)
+    HEXS_CASE(K_LINEAR)
 #undef HEXS_CASE
     default:
       return cudaErrorInvalidValue;
@@ -319,6 +354,13 @@ cudaError_t launch_naive_t(int kind, int dims, const NaiveArgs& a, cudaStream_t 
   }
   const T* src = static_cast<const T*>(a.src);
   T* dst = static_cast<T*>(a.dst);
+  if (kind == K_LINEAR) {
+    const int R = a.lin.R;
+    const int64_t X = dims == 3 ? N2 : N1, Y = dims == 3 ? N1 : N0;
+    dim3 grid((unsigned)((X - 2 * R + 255) / 256), (unsigned)(Y - 2 * R), dims == 3 ? (unsigned)(N0 - 2 * R) : 1u);
+    naive_linear_kernel<T><<<grid, 256, 0, s>>>(src, dst, N0, N1, dims == 3 ? N2 : 1, a.lin);
+    return cudaGetLastError();
+  }
   if (dims == 2) {
     dim3 grid((unsigned)((N1 - 2 + 255) / 256), (unsigned)((N0 - 2 + kNaiveStrip - 1) / kNaiveStrip));
     switch (kind) {

@@ -8,6 +8,15 @@ namespace hexs {
 
 constexpr int kMaxH = 64;
 
+// General linear stencil (K_LINEAR): acc = c_0 A[p+d_0]; acc = acc + c_k A[p+d_k] (left to
+// right), d_k the linear element offsets, over the interior [R, N-1-R] of every dimension.
+constexpr int kMaxLin = 64;
+struct LinearTerms {
+  int n, R;
+  int64_t delta[kMaxLin];
+  double coef[kMaxLin];
+};
+
 // Generic hybrid kernel (Table 4 configuration (a): hybrid schedule, global memory only).
 struct GenericArgs {
   void* f[3];      // ping-pong: f[0], f[1]; FDTD: ex, ey, hz (in place)
@@ -29,6 +38,7 @@ struct GenericArgs {
   int64_t S0_hi;
   int* flags;                   // [nS0][n1][n2], zeroed before the launch
   unsigned long long* counter;  // work counter, zeroed before the launch
+  LinearTerms lin;              // K_LINEAR: the access set and coefficients
 };
 cudaError_t launch_generic(int kind, int dtype, const GenericArgs& g, int grid, cudaStream_t s);
 // Persistent grid size of the wavefront kernel (all CTAs co-resident).
@@ -42,6 +52,7 @@ struct NaiveArgs {
   int64_t N[3];
   double k0, k1;
   int stmt;    // FDTD statement 0 = ey, 1 = ex, 2 = hz
+  LinearTerms lin;  // K_LINEAR
 };
 cudaError_t launch_naive(int kind, int dtype, int dims, const NaiveArgs& a, cudaStream_t s);
 

@@ -23,6 +23,24 @@ int fast2d_variant(int kind, int dtype, int h, int w0, int w1) {
   return -1;
 }
 
+int fast2d_variant_count() {
+  int n = 0;
+#define HEXS_CNT(id, dc, T_, KIND_, H_, W0_, NW_) ++n;
+  HEXS_FAST2D_VARIANTS(HEXS_CNT)
+#undef HEXS_CNT
+  return n;
+}
+bool fast2d_variant_info(int variant, int* kind, int* dtype, int* h, int* w0) {
+#define HEXS_INFO(id, dc, T_, KIND_, H_, W0_, NW_) \
+  if (variant == id) {                            \
+    *kind = KIND_; *dtype = dc; *h = H_; *w0 = W0_; \
+    return true;                                  \
+  }
+  HEXS_FAST2D_VARIANTS(HEXS_INFO)
+#undef HEXS_INFO
+  return false;
+}
+
 int fast2d_chunk_width(int variant) {
   switch (variant) {
 #define HEXS_W(id, dc, T_, KIND_, H_, W0_, NW_) case id: return fast2d_chunk_v##id();
@@ -60,6 +78,17 @@ int fast3d_variant(int kind, int dtype, int h, int w0, int wy) {
   HEXS_FAST3D_VARIANTS(HEXS_F3_MATCH)
 #undef HEXS_F3_MATCH
   return -1;
+}
+int fast3d_variant_count() { return HEXS_FAST3D_COUNT; }
+bool fast3d_variant_info(int variant, int* kind, int* dtype, int* h, int* w0) {
+#define HEXS_F3_INFO(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_) \
+  if (variant == id) {                                           \
+    *kind = KIND_; *dtype = dc; *h = H_; *w0 = W0_;              \
+    return true;                                                 \
+  }
+  HEXS_FAST3D_VARIANTS(HEXS_F3_INFO)
+#undef HEXS_F3_INFO
+  return false;
 }
 bool fast3d_variant_matches(int variant, int kind, int dtype, int h, int w0) {
 #define HEXS_F3_IS(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_) \

@@ -195,21 +195,21 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
       const int64_t slots = (int64_t)fdtd_ctas_per_sm() * device_sm_count();
       auto Wof = [&](int w) { return (int64_t)2 * w + 2 + h + h / 2; };
       while (w0 < 12 && (d.ext[0] + Wof(w0) - 1) / Wof(w0) + 1 > slots) ++w0;
-    } else if (d.dims == 2) {
-      // best measured on B200 (profiles/round1/tile_sweep_*.txt); the 9-point
-      // box takes the shallower hexagon: its unrolled level bodies otherwise overflow the
-      // instruction cache (ncu stall "no_instruction")
-      h = 3; w0 = 7;
-      if (d.kind == STENCIL_BOX2D9 && dtype == STENCIL_F32) h = 2;
-      // IEEE sqrt + div per point: only the smallest hexagon's body stays in the i-cache
-      if (d.kind == STENCIL_GRADIENT2D && dtype == STENCIL_F32) h = 1, w0 = 1;
     } else if (s3_class && p->hd == 1) {
       h = 2; w0 = 7;  // streaming kernel: Table 4's h = 2; two CTAs per SM
     } else {
-      h = 2; w0 = 7;  // Table 4 setup
-      // the 7-point star: one more level pair per tile amortises the per-tile fills and flags
-      // (measured 527 -> 550 GUp/s; profiles/round1/tile_sweep_heat3d.txt)
-      if (d.kind == STENCIL_STAR3D7 && dtype == STENCIL_F32) h = 3;
+      // the tile-size model (tilemodel.cpp: Sec. 3.7's load-to-compute ratio with the
+      // instruction-cache and CTA-count terms) over the compiled variants of the fast kernel
+      // that will run, or over modest hexagons for the generic executor
+      const bool unit = p->d0.n == 1 && p->d0.d == 1 && p->d1.n == 1 && p->d1.d == 1 && p->hd == 0;
+      int fam = FAMILY_GENERIC;
+      if (flags == STENCIL_EXEC_AUTO && unit && d.kind != STENCIL_LINEAR)
+        fam = d.dims == 2 ? FAMILY_FAST2D : FAMILY_FAST3D;
+      if (!tile_select(d, p->hd, p->d0, p->d1, fam, &h, &w0) &&
+          !tile_select(d, p->hd, p->d0, p->d1, FAMILY_GENERIC, &h, &w0)) {
+        h = 2;
+        w0 = 7;  // Table 4 setup
+      }
     }
   }
   if (h < 0 || w0 < 0) return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_plan: negative tile parameter");

@@ -24,6 +24,23 @@ static stencil_status cuda_fail(cudaError_t e, const char* where) {
     if (e_ != cudaSuccess) return cuda_fail(e_, where); \
   } while (0)
 
+// K_LINEAR terms: element offsets of the access set in the descriptor's order
+static void fill_linear(const Desc& d, LinearTerms& L) {
+  L = LinearTerms{};
+  if (d.kind != STENCIL_LINEAR) return;
+  L.n = (int)d.lcoef.size();
+  L.R = d.radius;
+  int64_t st[3] = {1, 1, 1};
+  st[d.dims - 1] = 1;
+  for (int q = d.dims - 2; q >= 0; --q) st[q] = st[q + 1] * d.ext[q + 1];
+  for (int k = 0; k < L.n; ++k) {
+    int64_t delta = 0;
+    for (int q = 0; q < d.dims; ++q) delta += (int64_t)d.loff[k * d.dims + q] * st[q];
+    L.delta[k] = delta;
+    L.coef[k] = d.lcoef[k];
+  }
+}
+
 static void fill_generic(const Plan& p, const Launch& l, GenericArgs& g) {
   const Desc& d = p.desc;
   g.dims = d.dims;
@@ -51,6 +68,7 @@ static void fill_generic(const Plan& p, const Launch& l, GenericArgs& g) {
     g.lo[a] = p.lo[a];
     g.hi[a] = p.hi[a];
   }
+  fill_linear(d, g.lin);
 }
 
 Plan::~Plan() {
@@ -112,6 +130,7 @@ stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* 
     for (int q = 0; q < 3; ++q) a.N[q] = q < d.dims ? d.ext[q] : 1;
     a.k0 = d.coef[0];
     a.k1 = d.coef[1];
+    fill_linear(d, a.lin);
     for (int f = 0; f < d.nfields; ++f) a.f[f] = out[f];
     for (int64_t tau = 0; tau < p.tau_levels; ++tau) {
       a.src = buf[tau & 1];

@@ -17,7 +17,7 @@ namespace hexs {
 
 enum Kind : int {
   K_JACOBI2D5 = 0, K_STAR2D5 = 1, K_BOX2D9 = 2, K_FDTD2D = 3,
-  K_STAR3D7 = 4, K_GRADIENT3D = 5, K_BOX3D27 = 6, K_GRADIENT2D = 7
+  K_STAR3D7 = 4, K_GRADIENT3D = 5, K_BOX3D27 = 6, K_GRADIENT2D = 7, K_LINEAR = 8
 };
 
 template <typename T> struct Coef { T k0, k1; };

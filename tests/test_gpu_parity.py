@@ -262,3 +262,31 @@ def test_output_tensors_validated():
     for o in bad:
         with pytest.raises(StencilError):
             plan.run(g, o)
+
+
+LIN_CASES = [
+    # 13-point star of radius 2, upwind (one-sided) of radius 2, a 3D radius-2 access set, and
+    # the 19-point 3D star-plus-edges of radius 1
+    ([(0, 0), (-1, 0), (1, 0), (0, -1), (0, 1), (-2, 0), (2, 0), (0, -2), (0, 2)],
+     [0.5, 0.1, 0.1, 0.1, 0.1, 0.025, 0.025, 0.025, 0.025], (67, 130), 13),
+    ([(0, 0), (0, -1), (0, -2), (-1, 0)], [0.25, 0.5, 0.125, 0.125], (50, 75), 11),
+    ([(0, 0, 0), (-2, 0, 0), (2, 0, 0), (0, -1, 0), (0, 1, 0), (0, 0, -2), (0, 0, 2), (1, 1, 1)],
+     [0.3, 0.1, 0.1, 0.1, 0.1, 0.1, 0.1, 0.1], (19, 21, 26), 7),
+    ([(0, 0, 0)] + [o for o in __import__("itertools").product((-1, 0, 1), repeat=3) if 0 < sum(map(abs, o)) <= 2],
+     [0.25] + [0.75 / 18] * 18, (17, 20, 23), 6),
+]
+
+
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("executor", ["auto", "naive"])
+@pytest.mark.parametrize("case", range(len(LIN_CASES)))
+def test_linear_stencils(case, executor, dtype):
+    """General linear stencils (any access set and radius: general delta, the generic hybrid
+    executor and the naive comparator) bit-exact against the oracle's plain loop."""
+    offs, coefs, shape, T = LIN_CASES[case]
+    g = stencil_inputs.uniform(shape, seed=40 + case, dtype=dtype)
+    st = Stencil("linear", shape, dtype=dtype, offsets=offs, coefficients=coefs)
+    plan = Plan(st, T, executor=executor)
+    out = plan.run(torch.from_numpy(g).cuda())
+    torch.cuda.synchronize()
+    assert_bitexact(out.cpu().numpy(), oracle.linear(g, offs, coefs, T), f"linear case {case} {executor}")
