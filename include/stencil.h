@@ -140,14 +140,15 @@ stencil_status stencil_run(stencil_plan_t plan, const void *const *in, void *con
  * Multi-GPU slab mode.  One process per GPU; the outermost grid
  * dimension (part_dim = 0: contiguous planes) is split evenly over the ranks.  Rank q owns
  * planes [own_lo, own_hi) and stores the local slab [loc_lo, loc_hi) = its owned planes plus
- * G = radius * D ghost planes on every side that is not a global boundary.  Time advances in
- * blocks of D steps, D a multiple of the hexagon height 2h+2 ("halos of width radius x
- * time-tile depth, exchanged once per time tile"); a block is the single-GPU hybrid schedule
- * of Sec. 3.6 over the local slab, whose outermost ghost plane stays
- * fixed -- after D steps every owned plane is exact (the dependence cone of an owned point over
- * D steps reaches radius * D planes), ghost planes are the only redundant work.  Between
- * blocks the library exchanges the ghost planes with rank +-1 by ncclSend / ncclRecv (one NCCL
- * group per block) on an internal stream ordered against the caller's stream by events.
+ * G = radius * (2h+2) ghost planes on every side that is not a global boundary ("halos of
+ * width radius x time-tile depth").  Every rank runs the GLOBAL run's launch table of the
+ * hybrid schedule (Sec. 3.6; hexagon tiling translated to the slab) over its
+ * slab, and before every launch but the first the library refreshes the ghost planes of both
+ * ping-pong buffers from rank +-1 by ncclSend / ncclRecv (one NCCL group per buffer) on an
+ * internal stream ordered against the caller's stream by events.  The slab's outermost planes
+ * stay fixed; a launch spans at most 2h+2 levels, so wrong values never travel past the ghost
+ * planes and every owned plane is exact after every launch; the ghost planes are the only
+ * redundant work, and the schedule is continuous (no time-block cuts).
  * NCCL is loaded at run time (the libnccl.so.2 the process already maps, e.g. PyTorch's;
  * environment HEXS_NCCL_LIB overrides); single-GPU use never needs it.  FDTD-2D is not
  * supported (STENCIL_E_UNSUPPORTED).
@@ -160,8 +161,9 @@ typedef struct {
   int64_t own_lo, own_hi; /* owned global planes of dimension 0                              */
   int64_t loc_lo, loc_hi; /* global planes held by the local slab                            */
   int64_t ghost;          /* G = radius * time_block                                         */
-  int64_t time_block;     /* D: steps between halo exchanges                                 */
-  int64_t n_blocks;       /* ceil(T_steps / D)                                               */
+  int64_t time_block;     /* 2h+2: levels a launch spans (the halo's time-tile depth)         */
+  int64_t n_blocks;       /* stencil_dist_info: launches per run (an exchange before each but
+                             the first); stencil_dist_layout: 0                               */
   int32_t h;              /* hexagon half-height the time block is a multiple of             */
   double ghost_fraction;  /* (local - owned) / owned planes: the redundant work              */
   int64_t launches_per_run; /* phase-kernel launches of one stencil_run (stencil_dist_info) */
@@ -190,12 +192,19 @@ stencil_status stencil_plan_dist(stencil_plan_t *out, stencil_desc_t global_desc
                                  const stencil_tile_t *tile, const void *nccl_unique_id, int rank,
                                  int nranks, int part_dim);
 
+/* Host-only: rank `rank`'s local plan -- the plan stencil_plan_dist runs on the slab (extent
+ * loc_hi - loc_lo along dimension 0, the global hexagon tiling kept) -- as an ordinary plan
+ * (introspection: launch table, schedule_of; or a single-GPU run of one rank's slab without
+ * halo exchanges).  Destroy it with stencil_destroy. */
+stencil_status stencil_dist_local_plan(stencil_plan_t *out, stencil_desc_t global_desc, int64_t T_steps,
+                                       const stencil_tile_t *tile, int rank, int nranks, int part_dim);
+
 /* The layout of a distributed plan and its launches per run. */
 stencil_status stencil_dist_info(stencil_plan_t plan, stencil_dist_info_t *info);
 
-/* A borrowed handle to the index-th local block plan of a distributed plan (0 = the D-step
- * plan; the last one may be a shorter remainder) -- for introspection and per-launch profiling
- * (stencil_plan_profile).  Owned by the distributed plan: never pass it to stencil_destroy. */
+/* A borrowed handle to the local plan of a distributed plan (index 0) -- for introspection and
+ * kernel-region profiling (stencil_plan_profile).  Owned by the distributed plan: never pass it
+ * to stencil_destroy. */
 stencil_status stencil_dist_block_plan(stencil_plan_t plan, int index, stencil_plan_t *block);
 
 /* Destroy a descriptor or plan (tagged handles).  NULL is a no-op.  A plan keeps its own

@@ -28,7 +28,7 @@ SYMBOLS = ["stencil_desc_create", "stencil_desc_deps", "stencil_plan",
            "stencil_plan_launches", "stencil_plan_hexagon", "stencil_plan_schedule_of",
            "stencil_plan_profile", "stencil_plan_profile_read", "stencil_abi_version",
            "stencil_dist_unique_id", "stencil_dist_layout", "stencil_plan_dist", "stencil_dist_info",
-           "stencil_dist_block_plan", "stencil_tile_model"]
+           "stencil_dist_block_plan", "stencil_tile_model", "stencil_dist_local_plan"]
 
 
 class StencilError(RuntimeError):
@@ -116,6 +116,7 @@ def lib() -> ctypes.CDLL:
     L.stencil_plan_dist.argtypes = [P(vp), vp, i64, P(Tile), vp, ctypes.c_int, ctypes.c_int, ctypes.c_int]
     L.stencil_dist_info.argtypes = [vp, P(DistInfo)]
     L.stencil_dist_block_plan.argtypes = [vp, ctypes.c_int, P(vp)]
+    L.stencil_dist_local_plan.argtypes = [P(vp), vp, i64, P(Tile), ctypes.c_int, ctypes.c_int, ctypes.c_int]
     L.stencil_tile_model.argtypes = [vp, ctypes.c_int, ctypes.c_int, ctypes.c_int, ctypes.c_int, P(TileEval)]
     for name in SYMBOLS:
         f = getattr(L, name)

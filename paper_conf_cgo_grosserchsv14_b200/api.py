@@ -91,6 +91,16 @@ class Plan:
         self._h = hp
         self._ws = None
 
+    @classmethod
+    def _adopt(cls, stencil: "Stencil", handle, T_steps: int) -> "Plan":
+        """Wrap a plan handle created elsewhere in the library (e.g. a slab's local plan)."""
+        p = cls.__new__(cls)
+        p.stencil = stencil
+        p.T_steps = int(T_steps)
+        p._h = handle
+        p._ws = None
+        return p
+
     # ---- introspection --------------------------------------------------------------
     @property
     def info(self) -> Dict[str, object]:

@@ -1,22 +1,24 @@
 // dist.cpp -- multi-GPU slab mode of the C ABI: one process per GPU,
 // the outermost grid dimension slab-partitioned over the ranks, halos exchanged with NCCL
-// send/recv over NVLink once per time block.
+// send/recv over NVLink once per phase launch (time tile).
 //
 // The paper's method is single-GPU: its host loop iterates the two phase kernels over the
-// whole grid (Sec. 4.1).  Scaling it over ranks keeps that hybrid schedule
-// unchanged inside every rank and adds overlapped tiling at rank edges only:
+// whole grid (Sec. 4.1).  Here every rank runs exactly that host loop -- the
+// SAME launch table (T, p) as the global run -- over its local slab, and the ranks exchange
+// halos between consecutive launches:
 //   * rank q owns planes [own_lo, own_hi) of dimension 0 (an even split) and stores the local
-//     slab [loc_lo, loc_hi) = owned planes plus G = radius * D ghost planes on every side that
-//     is not a global boundary;
-//   * time advances in blocks of D steps (D a multiple of the hexagon height 2h+2: the halos
-//     have the width "radius x time-tile depth" and are exchanged once per time tile);
-//   * a block is one stencil_run of a local single-GPU plan (the hybrid schedule over the slab,
-//     its outermost ghost plane held fixed): after D steps every owned plane is exact, because
-//     the dependence cone of an owned point over D steps reaches radius * D planes (the only
-//     redundant work is the ghost planes, 2G / owned of the compute);
-//   * between blocks the ghost planes are refreshed from the neighbours' owned planes:
-//     ncclGroupStart; ncclSend / ncclRecv to rank - 1 and rank + 1; ncclGroupEnd, on a
-//     communication stream ordered against the compute stream by events.
+//     slab [loc_lo, loc_hi) = owned planes plus G = radius * (2h+2) ghost planes on every side
+//     that is not a global boundary (the halo width "radius x time-tile depth");
+//   * the local plan keeps the GLOBAL hexagon tiling (when dimension 0 is the hexagonal one,
+//     its rows are translated by loc_lo -- Sec. 4.2.3's tile translation offset), so after every
+//     launch each plane of the slab holds the same levels as in a single-GPU run;
+//   * before every launch but the first, the ghost planes of BOTH ping-pong buffers are
+//     refreshed from the neighbours' owned planes (ncclGroupStart; ncclSend / ncclRecv to
+//     rank -1 and rank +1; ncclGroupEnd), on a communication stream ordered against the compute
+//     stream by events; the outermost local planes act as fixed (Dirichlet) planes, and a launch
+//     spans at most 2h+2 levels, so its wrong values never travel further than G planes: every
+//     owned plane is exact after every launch.  The only redundant work is the ghost planes
+//     (2G / owned of the compute); there are no time-block cuts (the schedule is continuous).
 // NCCL is loaded at run time (dlopen of the libnccl.so.2 the process already uses, e.g.
 // PyTorch's), so single-GPU use of the library never needs it; PyTorch only broadcasts the
 // 128-byte unique id (stencil_dist_unique_id on rank 0).
@@ -103,8 +105,8 @@ Plan* as_plan(stencil_plan_t h) {
 
 struct DistState {
   DistLayout lay;
-  std::vector<int64_t> blocks;                     // block lengths (D, ..., remainder)
-  std::vector<std::pair<int64_t, Plan*>> bplans;   // one local plan per distinct block length
+  std::vector<int64_t> blocks;                     // (one entry: T_steps; kept for the API)
+  std::vector<std::pair<int64_t, Plan*>> bplans;   // the local plan (one, T_steps long)
   Desc local;                                      // descriptor of the local slab
   size_t plane_bytes = 0;                          // bytes of one plane of dimension 0
   void* comm = nullptr;                            // ncclComm_t
@@ -151,16 +153,26 @@ void dist_fill_info(const Plan& p, stencil_plan_info_t& o) {
   o.workspace_bytes = p.ws_bytes;
 }
 
-// The tile of the local block plans: the caller's, else (3D) the (2, 7) hexagon -- a 6-step time
-// tile keeps the ghost planes of a 128-plane slab under 10% -- else the class default.
+// The tile of the local plans: the caller's, else (3D) the (2, 7) hexagon -- a 6-level time tile
+// keeps the ghost planes of a 128-plane slab under 10% -- else the class default the planner
+// picks for the GLOBAL grid.  Always returned explicit (h, w0), so every rank's local plan and the
+// layout share one hexagon (one tiling).
 stencil_tile_t dist_local_tile(const Desc& d, const stencil_tile_t* tile) {
   stencil_tile_t lt{};
   lt.hex_dim = -1;
   if (tile) lt = *tile;
   if (lt.h || lt.w0) return lt;  // an explicit hexagon
-  if (d.dims == 3 && (lt.flags == STENCIL_EXEC_AUTO)) {
+  if (d.dims == 3 && lt.flags == STENCIL_EXEC_AUTO) {
     lt.h = 2;
     lt.w0 = 7;
+    return lt;
+  }
+  Plan* probe = nullptr;
+  if (build_plan(d, 1, &lt, &probe) == STENCIL_OK) {
+    lt.h = probe->h;
+    lt.w0 = probe->w0;
+    if (lt.hex_dim < 0) lt.hex_dim = probe->hd;
+    delete probe;
   }
   return lt;
 }
@@ -186,29 +198,18 @@ stencil_status dist_layout(const Desc& d, int64_t T_steps, const stencil_tile_t*
   // by default, more while the ghost planes stay within ~10% of the owned ones);
   // HEXS_TIME_BLOCK overrides
   const stencil_tile_t lt = dist_local_tile(d, tile);
-  int h = lt.h;
-  if (!(lt.h || lt.w0)) {  // the class's automatic tile: ask the planner
-    Plan* probe = nullptr;
-    if (build_plan(d, 1, &lt, &probe) != STENCIL_OK) return STENCIL_E_INVALID;
-    h = probe->h;
-    delete probe;
-  }
+  const int h = lt.h;
   const int64_t H = 2 * (int64_t)h + 2;
   const int64_t owned = L.own_hi - L.own_lo;
-  int64_t D = H * std::max<int64_t>(1, owned / (20 * H));
-  if (const char* e = std::getenv("HEXS_TIME_BLOCK")) {
-    const int64_t v = std::atoll(e);
-    if (v > 0) D = v;
-  }
-  if (T_steps > 0) D = std::min(D, T_steps);
-  D = std::max<int64_t>(D, 1);
+  // one exchange per phase launch: a launch spans at most 2h+2 levels (one time tile)
+  const int64_t D = 2 * (int64_t)h + 2;
   L.time_block = D;
   L.ghost = (int64_t)d.radius * D;
   if (nranks > 1 && owned < L.ghost)
-    return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_plan_dist: a slab is thinner than the ghost width radius*D");
+    return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_plan_dist: a slab is thinner than the ghost width radius*(2h+2)");
   L.loc_lo = std::max<int64_t>(0, L.own_lo - L.ghost);
   L.loc_hi = std::min<int64_t>(N0, L.own_hi + L.ghost);
-  L.n_blocks = T_steps == 0 ? 0 : (T_steps + D - 1) / D;
+  L.n_blocks = 0;  // filled by stencil_plan_dist: launches (one exchange before each but the first)
   L.h = h;
   L.ghost_fraction = owned > 0 ? (double)((L.loc_hi - L.loc_lo) - owned) / (double)owned : 0.0;
   *out = L;
@@ -260,6 +261,17 @@ static stencil_status exchange(DistState& s, char* base, cudaStream_t stream) {
   return STENCIL_OK;
 }
 
+// pre_launch hook of the local plan: refresh both buffers' ghost planes
+static stencil_status ghost_hook(void* ctx, int64_t /*k*/, void* const* bufs, void* stream) {
+  DistState& s = *static_cast<DistState*>(ctx);
+  if (s.lay.nranks <= 1 || s.emulate) return STENCIL_OK;
+  for (int b = 0; b < 2; ++b) {
+    stencil_status st = exchange(s, static_cast<char*>(bufs[b]), static_cast<cudaStream_t>(stream));
+    if (st != STENCIL_OK) return st;
+  }
+  return STENCIL_OK;
+}
+
 stencil_status run_dist(Plan& p, const void* const* in, void* const* out, void* stream_) {
   DistState& s = *p.dist;
   cudaStream_t stream = static_cast<cudaStream_t>(stream_);
@@ -269,22 +281,13 @@ stencil_status run_dist(Plan& p, const void* const* in, void* const* out, void* 
   int dev = -1;
   if (cudaGetDevice(&dev) != cudaSuccess || dev != s.comm_dev)
     return fail(STENCIL_E_CUDA, "stencil_run: a distributed plan runs on the device it was created on");
-  const size_t bytes = (size_t)(s.lay.loc_hi - s.lay.loc_lo) * s.plane_bytes;
-  if (in[0] != out[0]) {
-    cudaError_t e = cudaMemcpyAsync(out[0], in[0], bytes, cudaMemcpyDeviceToDevice, stream);
-    if (e != cudaSuccess) return fail(STENCIL_E_CUDA, std::string("stencil_run: copy in->out: ") + cudaGetErrorString(e));
-  }
-  void* const* io = out;  // every block runs in place on the caller's output slab
-  for (size_t k = 0; k < s.blocks.size(); ++k) {
-    if (k > 0 && s.lay.nranks > 1 && !s.emulate) {
-      stencil_status st = exchange(s, static_cast<char*>(out[0]), stream);
-      if (st != STENCIL_OK) return st;
-    }
-    Plan* bp = s.plan_for(s.blocks[k]);
-    stencil_status st = run_plan(*bp, reinterpret_cast<const void* const*>(io), io, stream);
-    if (st != STENCIL_OK) return st;
-  }
-  return STENCIL_OK;
+  Plan* lp = s.bplans.empty() ? nullptr : s.bplans[0].second;
+  if (!lp) return STENCIL_OK;
+  lp->pre_launch = ghost_hook;
+  lp->pre_launch_ctx = &s;
+  // the local plan copies in -> out and runs the global launch table over the slab, exchanging
+  // the ghost planes before every launch but the first
+  return run_plan(*lp, in, out, stream);
 }
 
 }  // namespace hexs
@@ -355,14 +358,25 @@ stencil_status stencil_plan_dist(stencil_plan_t* out, stencil_desc_t global_desc
   if (s->local.ext[0] < 3) return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_plan_dist: local slab thinner than 3 planes");
   s->plane_bytes = d->elem();
   for (int q = 1; q < d->dims; ++q) s->plane_bytes *= (size_t)d->ext[q];
-  for (int64_t t = 0; t < T_steps; t += L.time_block) s->blocks.push_back(std::min(L.time_block, T_steps - t));
+  s->blocks.push_back(T_steps);
   const stencil_tile_t lt = dist_local_tile(*d, tile);
-  for (int64_t len : s->blocks) {
-    if (s->plan_for(len)) continue;
-    Plan* bp = nullptr;
-    st = build_plan(s->local, len, &lt, &bp);
+  {
+    // the local plan: the global schedule restricted to the slab (hexagon rows translated by
+    // loc_lo when dimension 0 is the hexagonal one, so the tiling matches the global one)
+    Plan* probe = nullptr;
+    st = build_plan(s->local, T_steps, &lt, &probe);
     if (st != STENCIL_OK) return st;
-    s->bplans.push_back({len, bp});
+    const int64_t origin = probe->hd == 0 ? L.loc_lo : 0;
+    delete probe;
+    Plan* bp = nullptr;
+    st = build_plan(s->local, T_steps, &lt, &bp, origin);
+    if (st != STENCIL_OK) return st;
+    if (bp->h != L.h) {
+      delete bp;
+      return fail(STENCIL_E_INVALID, "stencil_plan_dist: local tile differs from the layout's");
+    }
+    s->lay.n_blocks = (int64_t)bp->launches.size();
+    s->bplans.push_back({T_steps, bp});
   }
   // NCCL communicator and the communication stream on the current device
   if (cudaGetDevice(&s->comm_dev) != cudaSuccess) return fail(STENCIL_E_CUDA, "stencil_plan_dist: no CUDA device");
@@ -403,6 +417,32 @@ stencil_status stencil_plan_dist(stencil_plan_t* out, stencil_desc_t global_desc
   for (auto& bp : s->bplans) ws = std::max(ws, bp.second->ws_bytes);
   p->ws_bytes = ws;
   p->dist = s.release();
+  *out = reinterpret_cast<stencil_plan_t>(p);
+  return STENCIL_OK;
+}
+
+stencil_status stencil_dist_local_plan(stencil_plan_t* out, stencil_desc_t global_desc, int64_t T_steps,
+                                       const stencil_tile_t* tile, int rank, int nranks, int part_dim) {
+  clear_error();
+  if (!out) return fail(STENCIL_E_INVALID, "stencil_dist_local_plan: out is NULL");
+  *out = nullptr;
+  Desc* d = reinterpret_cast<Desc*>(global_desc);
+  if (!d || d->magic != kDescMagic) return fail(STENCIL_E_INVALID, "stencil_dist_local_plan: bad descriptor");
+  DistLayout L{};
+  stencil_status st = dist_layout(*d, T_steps, tile, rank, nranks, part_dim, &L);
+  if (st != STENCIL_OK) return st;
+  Desc local = *d;
+  local.ext[0] = L.loc_hi - L.loc_lo;
+  if (local.ext[0] < 3) return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_dist_local_plan: slab thinner than 3 planes");
+  const stencil_tile_t lt = dist_local_tile(*d, tile);
+  Plan* probe = nullptr;
+  st = build_plan(local, T_steps, &lt, &probe);
+  if (st != STENCIL_OK) return st;
+  const int64_t origin = probe->hd == 0 ? L.loc_lo : 0;
+  delete probe;
+  Plan* p = nullptr;
+  st = build_plan(local, T_steps, &lt, &p, origin);
+  if (st != STENCIL_OK) return st;
   *out = reinterpret_cast<stencil_plan_t>(p);
   return STENCIL_OK;
 }

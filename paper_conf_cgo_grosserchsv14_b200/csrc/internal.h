@@ -98,6 +98,11 @@ struct Plan {
   int ctrans[2] = {0, 0};  // classical tile translation offsets (Sec. 4.2.3)
   int h = 0, w0 = 0, w[2] = {1, 1};
   int H = 0, W = 0, F0 = 0, F1 = 0, c = 0;
+  int64_t hex_origin = 0;  // global coordinate of local row 0 along hd (slab plans)
+  // called before every phase-kernel launch k >= 1 with the two ping-pong buffers (multi-GPU
+  // slab mode: the per-launch ghost exchange); nullptr = none
+  stencil_status (*pre_launch)(void* ctx, int64_t k, void* const* bufs, void* stream) = nullptr;
+  void* pre_launch_ctx = nullptr;
   std::vector<int32_t> lo, hi;  // hexagon rows per level a
   std::vector<Launch> launches;
   int executor = EXEC_GENERIC;
@@ -132,7 +137,10 @@ stencil_status fail(stencil_status s, const std::string& msg);
 void clear_error();
 
 // plan.cpp
-stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* tile, Plan** out);
+// hex_origin: the global coordinate of local row 0 along the hexagonal dimension -- a local plan
+// of a slab (multi-GPU) keeps the global hexagon tiling (Sec. 4.2.3's tile translation offset)
+stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* tile, Plan** out,
+                          int64_t hex_origin = 0);
 bool schedule_of(const Plan& p, int64_t tau, const int64_t* s, int64_t* sched);
 
 // run.cu

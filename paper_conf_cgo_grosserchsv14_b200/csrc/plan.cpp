@@ -112,11 +112,11 @@ bool schedule_of(const Plan& p, int64_t tau, const int64_t* s, int64_t* sched) {
     int64_t T, n, a;
     if (ph == 0) {
       T = floor_div(tau + p.h + 1, p.H);                    // eq. (2)
-      n = s0 + p.F0 + p.w0 + 1 + T * p.c;                    // eq. (3), floor(d0 h)
+      n = s0 + p.hex_origin + p.F0 + p.w0 + 1 + T * p.c;     // eq. (3), floor(d0 h)
       a = tau + p.h + 1 - T * p.H;
     } else {
       T = floor_div(tau, p.H);                               // eq. (4)
-      n = s0 + T * p.c;                                      // eq. (5)
+      n = s0 + p.hex_origin + T * p.c;                       // eq. (5)
       a = tau - T * p.H;
     }
     const int64_t S0 = floor_div(n, p.W), b = n - S0 * p.W;
@@ -141,13 +141,15 @@ bool schedule_of(const Plan& p, int64_t tau, const int64_t* s, int64_t* sched) {
   return false;
 }
 
-stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* tile, Plan** out) {
+stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* tile, Plan** out,
+                          int64_t hex_origin) {
   if (T_steps < 0) return fail(STENCIL_E_INVALID, "stencil_plan: T_steps < 0");
   Plan* p = new (std::nothrow) Plan();
   if (!p) return fail(STENCIL_E_OOM, "stencil_plan: out of host memory");
   std::unique_ptr<Plan> guard(p);
   p->desc = d;
   p->T_steps = T_steps;
+  p->hex_origin = hex_origin;
   p->tau_levels = T_steps * (int64_t)d.stmts.size();
   stencil_tile_t t{};
   t.hex_dim = -1;  // NULL tile: everything automatic
@@ -329,7 +331,7 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
         ln.a_lo = (int)std::max<int64_t>(0, -ln.tau0);
         ln.a_hi = (int)std::min<int64_t>(p->H - 1, L - 1 - ln.tau0);
         if (ln.a_lo > ln.a_hi) continue;
-        ln.row_off = T * p->c + (ph == 0 ? p->F0 + w0 + 1 : 0);
+        ln.row_off = T * p->c + (ph == 0 ? p->F0 + w0 + 1 : 0) + p->hex_origin;
         int bmin = INT32_MAX, bmax = INT32_MIN;
         for (int a = ln.a_lo; a <= ln.a_hi; ++a) {
           bmin = std::min(bmin, (int)p->lo[a]);

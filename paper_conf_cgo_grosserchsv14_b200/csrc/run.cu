@@ -147,7 +147,14 @@ stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* 
     if (p.executor == EXEC_STREAM3D)
       HEXS_CUDA(cudaMemsetAsync(static_cast<char*>(p.ws) + p.s3_ctr_off, 0, p.s3_ctr_bytes, s),
                 "stencil_run: reset strip progress counters");
+    int64_t launch_k = 0;
     for (const Launch& l : p.launches) {
+      if (p.pre_launch && launch_k > 0) {
+        void* const bufs[2] = {buf[0], buf[1]};
+        const stencil_status hs = p.pre_launch(p.pre_launch_ctx, launch_k, bufs, s);
+        if (hs != STENCIL_OK) return hs;
+      }
+      ++launch_k;
       const int a_final = (l.tau0 + l.a_hi + 1 == p.tau_levels) ? l.a_hi : -1;
       const int64_t grid64 = l.S0_hi - l.S0_lo + 1;
       if (grid64 > INT32_MAX) return fail(STENCIL_E_UNSUPPORTED, "stencil_run: grid too large");

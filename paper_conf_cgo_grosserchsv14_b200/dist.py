@@ -52,9 +52,6 @@ class Layout:
     def own_local(self) -> Tuple[int, int]:
         return self.own_lo - self.loc_lo, self.own_hi - self.loc_lo
 
-    def blocks(self, T: int) -> List[int]:
-        D = self.time_block
-        return [min(D, T - t) for t in range(0, T, D)]
 
 
 def _tile(h=0, w0=0, w=(0, 0, 0), hex_dim=-1, executor="auto") -> Tile:
@@ -90,6 +87,23 @@ def layout(kind: str, global_ext: Sequence[int], T: int, rank: int, nranks: int,
         lib().stencil_destroy(d)
 
 
+def local_plan(kind: str, global_ext: Sequence[int], T: int, rank: int, nranks: int, dtype="float32", **tile):
+    """Rank `rank`'s local plan (host only; stencil_dist_local_plan): the global launch table of
+    the hybrid schedule restricted to the slab -- what a distributed plan runs between its halo
+    exchanges."""
+    from .api import Plan, Stencil
+
+    lay = layout(kind, global_ext, T, rank, nranks, dtype, **tile)
+    d = _desc(kind, global_ext, dtype)
+    try:
+        h = ctypes.c_void_p()
+        t = _tile(**tile)
+        check(lib().stencil_dist_local_plan(ctypes.byref(h), d, int(T), ctypes.byref(t), int(rank), int(nranks), 0))
+    finally:
+        lib().stencil_destroy(d)
+    return Plan._adopt(Stencil(kind, lay.local_ext, dtype=dtype), h, T), lay
+
+
 def exchange_halos(local: torch.Tensor, lay: Layout, group=None) -> None:
     """The library's halo step over torch.distributed (for CPU/gloo tests of the protocol):
     send my first / last G owned planes down / up, receive the neighbours' into my ghosts."""
@@ -107,15 +121,15 @@ def exchange_halos(local: torch.Tensor, lay: Layout, group=None) -> None:
             req.wait()
 
 
-def run_protocol(local: torch.Tensor, lay: Layout, T: int, compute: Callable[[torch.Tensor, int], None],
-                 group=None) -> torch.Tensor:
-    """The distributed run of csrc/dist.cpp::run_dist with an injected per-block compute and a
-    torch.distributed exchange: for each block, exchange (but before the first), then D steps."""
-    for k, steps in enumerate(lay.blocks(T)):
+def run_protocol(bufs: Sequence[torch.Tensor], lay: Layout, plan, execute_launch: Callable, group=None) -> None:
+    """The distributed run of csrc/dist.cpp::run_dist with an injected launch executor and a
+    torch.distributed exchange: for each launch of the rank's local plan, refresh the ghost
+    planes of both ping-pong buffers (but before the first), then run the launch."""
+    for k, ln in enumerate(plan.launches()):
         if k > 0 and lay.nranks > 1:
-            exchange_halos(local, lay, group)
-        compute(local, steps)
-    return local
+            for b in bufs:
+                exchange_halos(b, lay, group)
+        execute_launch(ln, bufs)
 
 
 class DistPlan:

@@ -1,13 +1,16 @@
 """Multi-process (world_size 2 and 3, gloo backend, CPU) tests of the slab-mode protocol of the
 C ABI's distributed plans (csrc/dist.cpp, include/stencil.h stencil_plan_dist).  Each rank takes
-its layout from the library's host-only stencil_dist_layout (the exact partition, ghost width and
-time block stencil_plan_dist uses), runs the library's block loop (paper_conf_cgo_grosserchsv14_b200
-.dist.run_protocol: halo exchange between blocks, D steps per block on the local slab) with the
-CPU oracle injected as the per-block compute (there is no GPU here; on the GPU box the blocks run
-the hybrid kernels and the exchange is NCCL), and the gathered owned planes must be
+its layout and its local plan from the library's host-only stencil_dist_layout /
+stencil_dist_local_plan (the exact partition, ghost width and slab launch table -- the global
+hexagon tiling translated to the slab -- that stencil_plan_dist runs), then runs the library's
+loop (paper_conf_cgo_grosserchsv14_b200.dist.run_protocol: the ghost planes of both ping-pong
+buffers exchanged before every launch but the first) with a CPU executor of the launch table
+(tests/_schedexec.py) in place of the kernels (there is no GPU here; on the GPU box the launches
+are the hybrid kernels and the exchange is NCCL).  The gathered owned planes must be
 bit-identical to the single-domain oracle ("bit-identical for every P")."""
 import os
 import socket
+import sys
 
 import numpy as np
 import pytest
@@ -17,6 +20,9 @@ import torch.multiprocessing as mp
 
 import oracle
 import stencil_inputs
+
+sys.path.insert(0, os.path.dirname(os.path.abspath(__file__)))
+from paper_conf_cgo_grosserchsv14_b200 import Plan, Stencil
 from paper_conf_cgo_grosserchsv14_b200 import dist as hdist
 
 
@@ -28,40 +34,36 @@ def _free_port():
     return p
 
 
-def _worker(rank, world, port, kind, ext, T, block, out_dir):
+def _worker(rank, world, port, kind, ext, T, out_dir):
+    import _schedexec
+
     os.environ["MASTER_ADDR"] = "127.0.0.1"
     os.environ["MASTER_PORT"] = str(port)
-    if block:
-        os.environ["HEXS_TIME_BLOCK"] = str(block)
     dist.init_process_group("gloo", rank=rank, world_size=world)
     try:
-        lay = hdist.layout(kind, ext, T, rank, world)
-
-        def compute(local, steps):  # test-only injection of the CPU oracle (the local slab alone)
-            local.copy_(torch.from_numpy(oracle.run(kind, local.numpy(), steps)))
-
+        plan, lay = hdist.local_plan(kind, ext, T, rank, world)
         g = stencil_inputs.uniform(ext, seed=5)
-        local = torch.from_numpy(np.ascontiguousarray(g[lay.loc_lo:lay.loc_hi]))
-        assert tuple(local.shape) == lay.local_ext
-        hdist.run_protocol(local, lay, T, compute)
+        local = np.ascontiguousarray(g[lay.loc_lo:lay.loc_hi])
+        assert local.shape == lay.local_ext
+        bufs = [torch.from_numpy(local.copy()), torch.from_numpy(local.copy())]
+        ex = _schedexec.launch_executor(plan, kind)
+        hdist.run_protocol(bufs, lay, plan, lambda ln, b: ex(ln, [x.numpy() for x in b]))
         lo, hi = lay.own_local
-        np.save(os.path.join(out_dir, f"r{rank}.npy"), local[lo:hi].numpy())
+        np.save(os.path.join(out_dir, f"r{rank}.npy"), bufs[T % 2][lo:hi].numpy())
         np.save(os.path.join(out_dir, f"r{rank}_lo.npy"), np.array([lay.own_lo]))
     finally:
         dist.destroy_process_group()
 
 
-@pytest.mark.parametrize("kind,ext,T,block,world", [
-    ("star2d5", (41, 23), 17, 4, 2),
-    ("box2d9", (50, 19), 13, 5, 3),
-    ("jacobi2d5", (30, 30), 9, 0, 2),
-    ("star3d7", (22, 9, 11), 7, 3, 2),
-    ("star3d7", (40, 9, 12), 13, 0, 3),
-    ("gradient3d", (26, 8, 8), 8, 0, 2),
+@pytest.mark.parametrize("kind,ext,T,world", [
+    ("star2d5", (61, 23), 17, 2),
+    ("star2d5", (90, 19), 29, 3),
+    ("star3d7", (40, 9, 11), 13, 2),
+    ("star3d7", (44, 8, 10), 11, 3),
 ])
-def test_slab_mode_bit_identical(tmp_path, kind, ext, T, block, world):
+def test_slab_mode_bit_identical(tmp_path, kind, ext, T, world):
     port = _free_port()
-    mp.spawn(_worker, args=(world, port, kind, ext, T, block, str(tmp_path)), nprocs=world, join=True)
+    mp.spawn(_worker, args=(world, port, kind, ext, T, str(tmp_path)), nprocs=world, join=True)
     parts = []
     for r in range(world):
         lo = int(np.load(tmp_path / f"r{r}_lo.npy")[0])
@@ -71,6 +73,24 @@ def test_slab_mode_bit_identical(tmp_path, kind, ext, T, block, world):
     exp = oracle.run(kind, stencil_inputs.uniform(ext, seed=5), T)
     assert got.shape == exp.shape
     assert np.array_equal(got, exp)
+
+
+def test_local_plan_keeps_the_global_tiling():
+    """A slab's local plan is the global schedule translated by loc_lo: every instance of the
+    slab has the same (T, p, S0, t', s') as in the global plan (Sec. 4.2.3 translation)."""
+    ext, T = (61, 23), 17
+    gplan = None
+    for rank in range(3):
+        plan, lay = hdist.local_plan("star2d5", ext, T, rank, 3)
+        if gplan is None:  # the global plan with the slabs' hexagon
+            gplan = Plan(Stencil("star2d5", ext), T, h=plan.info["h"], w0=plan.info["w0"])
+        assert (plan.info["h"], plan.info["w0"], plan.info["W"]) == (gplan.info["h"], gplan.info["w0"], gplan.info["W"])
+        for tau in range(0, T, 3):
+            for r in range(0, lay.loc_hi - lay.loc_lo, 2):
+                for j in range(0, ext[1], 5):
+                    loc = plan.schedule_of(tau, (r, j))
+                    glob = gplan.schedule_of(tau, (r + lay.loc_lo, j))
+                    assert loc[:3] == glob[:3] and loc[4] == glob[4] and loc[5] == glob[5]
 
 
 def test_layout_properties():
@@ -91,10 +111,9 @@ def test_layout_properties():
                 assert a.own_hi == b.own_lo
             for lay in lays:
                 G = lay.ghost
-                assert G == lay.time_block
+                assert G == lay.time_block == 2 * lay.h + 2  # radius x time-tile depth
                 assert lay.loc_lo == max(0, lay.own_lo - G) and lay.loc_hi == min(N0, lay.own_hi + G)
                 assert lay.local_ext == (lay.loc_hi - lay.loc_lo, 40)
-                assert sum(lay.blocks(50)) == 50 and len(lay.blocks(50)) == lay.n_blocks
     for P in (2, 4, 8):
         for r in (0, P // 2, P - 1):
             lay = hdist.layout("star3d7", (1024, 1024, 1024), 256, r, P)
