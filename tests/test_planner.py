@@ -214,6 +214,8 @@ def test_naive_and_auto_executor_selection():
     p = Plan(Stencil("star2d5", (64, 64)), 8, executor="naive")
     assert p.info["executor"] == 2 and p.info["n_launches"] == 8
     p = Plan(Stencil("star2d5", (64, 64)), 8)
+    assert p.info["fast_kernel"] == 1  # a compiled variant, the tile model's choice for this grid
+    p = Plan(Stencil("star2d5", (8192, 8192)), 8)
     assert p.info["fast_kernel"] == 1 and p.info["h"] == 3 and p.info["w0"] == 7
     p = Plan(Stencil("star2d5", (64, 64)), 8, h=2, w0=2)   # no specialised instantiation
     assert p.info["fast_kernel"] == 0
