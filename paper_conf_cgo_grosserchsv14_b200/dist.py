@@ -257,7 +257,11 @@ def bench_main(args, cfg, configs, metric, helpers):
     if not dist.is_initialized():
         dist.init_process_group("nccl", device_id=torch.device("cuda", local_rank))
     gext = ((ext[0] * world,) + tuple(ext[1:])) if scaling == "weak" else tuple(ext)
-    dp = DistPlan(kind, gext, T)
+    tile = {}
+    if getattr(args, "tile", ""):  # h,w0: the local plans' hexagon (tuning)
+        v = [int(x) for x in args.tile.split(",")]
+        tile = {"h": v[0], "w0": v[1]}
+    dp = DistPlan(kind, gext, T, **tile)
     lay = dp.layout
     plane = 1
     for e in gext[1:]:
