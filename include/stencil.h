@@ -83,7 +83,18 @@ enum {
   STENCIL_EXEC_AUTO = 0,    /* fastest implemented hybrid-tiled kernel for the class      */
   STENCIL_EXEC_GENERIC = 1, /* generic hybrid kernel straight from global memory
                                (Table 4 configuration (a))                 */
-  STENCIL_EXEC_NAIVE = 2    /* non-time-tiled comparator: one launch per time step       */
+  STENCIL_EXEC_NAIVE = 2,   /* non-time-tiled comparator: one launch per time step       */
+  /* B200 replay of the optimisation ablation of Sec. 6.2 (Table 4): one 3D
+   * hybrid phase kernel (kernels/ablation.cu) with the paper's CTA of 1 x 10 x 32 threads and
+   * classical tiles w1 = 10, w2 = 32 (tile.w must be 0 or {10, 32}), hexagons over dimension 0,
+   * differing only in the memory strategy.  3D radius-1 single-field classes (star3d7, box3d27,
+   * gradient3d), STENCIL_F32 only (the paper's precision); anything else STENCIL_E_UNSUPPORTED. */
+  STENCIL_EXEC_T4A = 3, /* (a) no shared memory: operands and results in global memory       */
+  STENCIL_EXEC_T4B = 4, /* (b) copy-in box -> compute in shared memory -> copy-out phase      */
+  STENCIL_EXEC_T4C = 5, /* (c) (b) with interleaved copy-out (store as computed)              */
+  STENCIL_EXEC_T4D = 6, /* (d) (c) with tiles translated so the copy-in box is 128-B aligned  */
+  STENCIL_EXEC_T4E = 7, /* (e) (d) + static reuse: fixed smem home per value (x mod 64)        */
+  STENCIL_EXEC_T4F = 8  /* (f) (d) + dynamic reuse: explicit copy phase between x tiles        */
 };
 
 /* Create a stencil descriptor.
@@ -244,7 +255,8 @@ enum {
   STENCIL_KERNEL_FAST2D = 2,    /* 2D register wavefront, TMA-staged In rows                  */
   STENCIL_KERNEL_FDTD = 3,      /* FDTD-2D shared-memory ring                                 */
   STENCIL_KERNEL_FAST3D = 4,    /* 3D tile wavefront, hexagons over (t, z), levels in smem    */
-  STENCIL_KERNEL_STREAM3D = 5   /* 3D streaming: hexagons over (t, y), z streamed, registers  */
+  STENCIL_KERNEL_STREAM3D = 5,  /* 3D streaming: hexagons over (t, y), z streamed, registers  */
+  STENCIL_KERNEL_ABLATION = 6   /* Table 4 replay (STENCIL_EXEC_T4A..T4F)                      */
 };
 
 stencil_status stencil_plan_info(stencil_plan_t plan, stencil_plan_info_t *info);

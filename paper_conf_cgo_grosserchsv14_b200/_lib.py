@@ -19,7 +19,8 @@ STATUS = {0: "STENCIL_OK", 1: "STENCIL_E_INVALID", 2: "STENCIL_E_UNSUPPORTED",
 
 KINDS = {"jacobi2d5": 0, "star2d5": 1, "box2d9": 2, "fdtd2d": 3, "star3d7": 4,
          "gradient3d": 5, "box3d27": 6, "gradient2d": 7, "linear": 8}
-EXEC = {"auto": 0, "generic": 1, "naive": 2}
+EXEC = {"auto": 0, "generic": 1, "naive": 2,  # + the Table 4 replay (a)-(f)
+        "t4a": 3, "t4b": 4, "t4c": 5, "t4d": 6, "t4e": 7, "t4f": 8}
 
 # every symbol include/stencil.h declares
 SYMBOLS = ["stencil_desc_create", "stencil_desc_deps", "stencil_plan",
@@ -57,7 +58,7 @@ class PlanInfo(ctypes.Structure):
                 ("tile_in", ctypes.c_int64), ("tile_out", ctypes.c_int64),
                 ("workspace_bytes", ctypes.c_size_t), ("kernel", ctypes.c_int32)]
 
-KERNELS = {0: "generic", 1: "naive", 2: "fast2d", 3: "fdtd", 4: "fast3d", 5: "stream3d"}
+KERNELS = {0: "generic", 1: "naive", 2: "fast2d", 3: "fdtd", 4: "fast3d", 5: "stream3d", 6: "ablation"}
 
 
 class DistInfo(ctypes.Structure):

@@ -74,7 +74,8 @@ struct Launch {
   int64_t s3_ctr_first = 0;
 };
 
-enum Executor { EXEC_GENERIC = 1, EXEC_NAIVE = 2, EXEC_FAST2D = 3, EXEC_FDTD = 4, EXEC_FAST3D = 5, EXEC_STREAM3D = 6 };
+enum Executor { EXEC_GENERIC = 1, EXEC_NAIVE = 2, EXEC_FAST2D = 3, EXEC_FDTD = 4, EXEC_FAST3D = 5, EXEC_STREAM3D = 6,
+               EXEC_ABLATION = 7 };
 
 // Multi-GPU slab mode (dist.cpp): partition, time blocks, local block plans, NCCL state.
 struct DistLayout {

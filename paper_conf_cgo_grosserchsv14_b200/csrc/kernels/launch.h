@@ -124,4 +124,27 @@ struct Stream3DArgs {
 };
 cudaError_t launch_stream3d(int variant, const Stream3DArgs& a, cudaStream_t s);
 
+// Table 4 ablation kernel (kernels/ablation.cu): one hybrid 3D phase kernel per memory strategy
+// (a) global only .. (f) dynamic reuse, CTA 1 x 10 x 32 over classical tiles of 10 (y) x 32 (x).
+enum { ABL_A = 0, ABL_B = 1, ABL_C = 2, ABL_D = 3, ABL_E = 4, ABL_F = 5 };
+constexpr int kAblW1 = 10, kAblW2 = 32;
+struct AblArgs {
+  void* buf[2];
+  int64_t N0, N1, N2;
+  int64_t tau0;
+  int a_lo, a_hi;
+  int64_t S0_lo, S0_hi, row_off;
+  int W;
+  int64_t S1_lo, S2_lo;
+  int n1, n2;            // y tiles (rows of the pipeline) and x tiles per row
+  int ctrans1, ctrans2;  // classical translation offsets (tile bases B = S w + ctrans - a)
+  int YB, XB, XP;        // shared box: y lines, x columns loaded, x pitch (64 = circular)
+  double k0, k1;
+  int* progress;               // [n1][nS0] completed x tiles per row, zeroed per launch
+  unsigned int* counter;       // row ticket, zeroed per launch
+  int32_t lo[kMaxH], hi[kMaxH];
+};
+cudaError_t launch_ablation(int cfg, int kind, const AblArgs& a, cudaStream_t s);
+size_t ablation_smem_bytes(int cfg, int W, int YB, int XP);
+
 }  // namespace hexs

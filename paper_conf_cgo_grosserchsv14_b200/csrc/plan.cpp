@@ -183,11 +183,15 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
 
   // a2: tile parameters
   const int flags = t.flags;
+  const bool ablation = flags >= STENCIL_EXEC_T4A && flags <= STENCIL_EXEC_T4F;
   bool auto_tile = (t.h == 0 && t.w0 == 0);
   int h = t.h, w0 = t.w0;
   const int dtype = d.dtype;
   if (auto_tile) {
-    if (d.kind == STENCIL_FDTD2D) {
+    if (ablation) {
+      h = 2;
+      w0 = 7;  // Table 4's tile
+    } else if (d.kind == STENCIL_FDTD2D) {
       // 24 tau-levels = 8 full steps per tile (h+1 a multiple of 3, reading R14); w0 as
       // small as possible while every launch's hexagons (W = 2 w0 + 2 + h + h/2 rows) fit one
       // wave of the FDTD kernel (fdtd_ctas_per_sm() CTAs per SM): a second, partial wave would double the
@@ -278,6 +282,20 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
           p->d0.d == 1 && p->d1.n == 1 && p->d1.d == 1)
         ex = EXEC_FAST3D;
     }
+  } else if (ablation) {
+    // Table 4 replay: the 3D radius-1 single-field classes in fp32, hexagons over z, unit skews
+    if (d.dims != 3 || !(d.kind == STENCIL_STAR3D7 || d.kind == STENCIL_BOX3D27 || d.kind == STENCIL_GRADIENT3D) ||
+        d.dtype != STENCIL_F32 || p->hd != 0 || !(p->d0.n == 1 && p->d0.d == 1 && p->d1.n == 1 && p->d1.d == 1) ||
+        p->dcls[0] != 1 || p->dcls[1] != 1)
+      return fail(STENCIL_E_UNSUPPORTED,
+                  "stencil_plan: the Table 4 executors take 3D radius-1 star3d7/box3d27/gradient3d fp32, hex_dim 0");
+    if (!((t.w[0] == 0 && t.w[1] == 0) || (t.w[0] == 10 && t.w[1] == 32)))
+      return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_plan: the Table 4 executors use w = {10, 32} (PAPER.md:998-1000)");
+    ex = EXEC_ABLATION;
+    p->variant = flags - STENCIL_EXEC_T4A;
+    const int YB = p->H + 11, XB = p->H + 33, XP = p->variant == 4 ? 64 : XB;
+    if (XB > 64 || 2.0 * (p->W + 2) * YB * XP * 4 > 227.0 * 1024)
+      return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_plan: the Table 4 copy-in box exceeds shared memory");
   } else if (flags != STENCIL_EXEC_GENERIC) {
     return fail(STENCIL_E_INVALID, "stencil_plan: unknown tile.flags");
   }
@@ -287,6 +305,7 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
   for (int q = 0; q < p->ncls; ++q) {
     int wq = t.w[q];
     if (ex == EXEC_FAST2D) wq = fast2d_chunk_width(p->variant);
+    else if (ex == EXEC_ABLATION) wq = q == 0 ? 10 : 32;  // Table 4: w1 = 10, w2 = 32
     else if (ex == EXEC_STREAM3D) wq = q == 0 ? 1 : kStream3DNXPlan;  // z planes streamed; x strips
     else if (ex == EXEC_FAST3D) {
       int wy = 0, wx = 0;
@@ -306,6 +325,13 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
   if (ex == EXEC_FAST3D || ex == EXEC_STREAM3D) {
     p->dcls[1] = std::max(p->dcls[1], 4);
     p->ctrans[1] = 0;
+  }
+  // Table 4 (d)-(f) translate the x tiles (Sec. 4.2.3's offset): (d) so the
+  // copy-in box [B2 - H, B2 + 33) of a full launch starts on a 128-B line, (e)/(f) so the 32
+  // columns each later tile loads, [B2 + 1, B2 + 33), are one aligned line
+  if (ex == EXEC_ABLATION) {
+    p->ctrans[0] = 0;
+    p->ctrans[1] = p->variant == 3 ? p->H % 32 : (p->variant >= 4 ? 31 : 0);
   }
 
   // a3: launch table.  Order (T, 0), (T, 1), T ascending.
@@ -359,7 +385,7 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
   if (d.pingpong && T_steps > 0) p->ws_bytes = ((size_t)d.points() * d.elem() + 255) / 256 * 256;
   // 3D generic executor: classical tiles run as a dependence wavefront; per-tile completion
   // flags and a work counter follow the ping-pong buffer in the workspace.
-  p->wavefront = ((ex == EXEC_GENERIC || ex == EXEC_FAST3D) && d.dims == 3 && p->ncls == 2);
+  p->wavefront = ((ex == EXEC_GENERIC || ex == EXEC_FAST3D || ex == EXEC_ABLATION) && d.dims == 3 && p->ncls == 2);
   if (p->wavefront && !p->launches.empty()) {
     // every launch owns its flags and work counter, so one memset per stencil_run resets
     // them all (no reset between the launches of a run)
@@ -367,7 +393,9 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
     for (Launch& l : p->launches) {
       l.flag_first = n_items;
       l.counter_idx = idx++;
-      n_items += (l.S0_hi - l.S0_lo + 1) * (l.Shi[0] - l.Slo[0] + 1) * (l.Shi[1] - l.Slo[1] + 1);
+      // (the Table 4 kernel keeps one progress counter per (hexagon, y tile) row)
+      n_items += (l.S0_hi - l.S0_lo + 1) * (l.Shi[0] - l.Slo[0] + 1) *
+                 (ex == EXEC_ABLATION ? 1 : (l.Shi[1] - l.Slo[1] + 1));
     }
     p->flag_off = p->ws_bytes;
     p->counter_off = p->flag_off + ((size_t)n_items * sizeof(int) + 255) / 256 * 256;
@@ -479,14 +507,17 @@ stencil_status stencil_plan_info(stencil_plan_t plan, stencil_plan_info_t* info)
   o.W = p->W;
   o.F0 = p->F0;
   o.F1 = p->F1;
-  o.executor = p->executor == EXEC_NAIVE ? STENCIL_EXEC_NAIVE
-             : p->executor == EXEC_GENERIC ? STENCIL_EXEC_GENERIC : STENCIL_EXEC_AUTO;
+  o.executor = p->executor == EXEC_NAIVE       ? STENCIL_EXEC_NAIVE
+               : p->executor == EXEC_GENERIC   ? STENCIL_EXEC_GENERIC
+               : p->executor == EXEC_ABLATION ? STENCIL_EXEC_T4A + p->variant
+                                               : STENCIL_EXEC_AUTO;
   o.fast_kernel = (p->executor == EXEC_FAST2D || p->executor == EXEC_FDTD || p->executor == EXEC_FAST3D ||
                    p->executor == EXEC_STREAM3D);
   o.kernel = p->executor == EXEC_FAST2D ? STENCIL_KERNEL_FAST2D
            : p->executor == EXEC_FDTD ? STENCIL_KERNEL_FDTD
            : p->executor == EXEC_FAST3D ? STENCIL_KERNEL_FAST3D
            : p->executor == EXEC_STREAM3D ? STENCIL_KERNEL_STREAM3D
+           : p->executor == EXEC_ABLATION ? STENCIL_KERNEL_ABLATION
            : p->executor == EXEC_NAIVE ? STENCIL_KERNEL_NAIVE : STENCIL_KERNEL_GENERIC;
   o.n_launches = p->executor == EXEC_NAIVE ? p->tau_levels : (int64_t)p->launches.size();
   o.T_steps = p->T_steps;

@@ -220,6 +220,40 @@ stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* 
         a.ticket = reinterpret_cast<unsigned int*>(a.progress + a.n_items);
         a.scratch = reinterpret_cast<float*>(ws + p.s3_scratch_off);
         HEXS_CUDA(launch_stream3d(p.variant, a, s), "stencil_run: stream3d kernel launch");
+      } else if (p.executor == EXEC_ABLATION) {
+        AblArgs a{};
+        a.buf[0] = buf[0];
+        a.buf[1] = buf[1];
+        a.N0 = d.ext[0];
+        a.N1 = d.ext[1];
+        a.N2 = d.ext[2];
+        a.tau0 = l.tau0;
+        a.a_lo = l.a_lo;
+        a.a_hi = l.a_hi;
+        a.S0_lo = l.S0_lo;
+        a.S0_hi = l.S0_hi;
+        a.row_off = l.row_off;
+        a.W = p.W;
+        a.S1_lo = l.Slo[0];
+        a.S2_lo = l.Slo[1];
+        a.n1 = (int)(l.Shi[0] - l.Slo[0] + 1);
+        a.n2 = (int)(l.Shi[1] - l.Slo[1] + 1);
+        a.ctrans1 = p.ctrans[0];
+        a.ctrans2 = p.ctrans[1];
+        a.YB = p.H + 11;
+        a.XB = p.H + 33;
+        a.XP = p.variant == ABL_E ? 64 : a.XB;
+        a.k0 = d.coef[0];
+        a.k1 = d.coef[1];
+        for (int q = 0; q < p.H; ++q) {
+          a.lo[q] = p.lo[q];
+          a.hi[q] = p.hi[q];
+        }
+        char* ws = static_cast<char*>(p.ws);
+        a.progress = reinterpret_cast<int*>(ws + p.flag_off) + l.flag_first;
+        a.counter = reinterpret_cast<unsigned int*>(reinterpret_cast<unsigned long long*>(ws + p.counter_off) +
+                                                    l.counter_idx);
+        HEXS_CUDA(launch_ablation(p.variant, d.kind, a, s), "stencil_run: Table 4 kernel launch");
       } else if (p.executor == EXEC_FAST3D) {
         Fast3DArgs a{};
         a.buf[0] = buf[0];

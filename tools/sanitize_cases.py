@@ -82,6 +82,9 @@ CASES = {
     "fdtd": ("fdtd2d", (60, 136), 9, np.float32, 0, 0),
     "generic3d": ("star3d7", (18, 21, 23), 6, np.float32, 1, 1),
 }
+# Table 4 replay (kernels/ablation.cu): every memory strategy, 2 x tiles per row and 2 y rows
+for _c in "abcdef":
+    CASES[f"t4{_c}"] = ("box3d27", (24, 22, 70), 7, np.float32, 0, 0)
 
 
 def main(argv):
@@ -89,8 +92,8 @@ def main(argv):
     bad = []
     for n in names:
         kind, shape, T, dt, h, w0 = CASES[n]
-        ex = "generic" if n.startswith("generic") else "auto"
-        hd = 0 if n.startswith("fast3d") else (1 if n.startswith("stream3d") else -1)
+        ex = "generic" if n.startswith("generic") else (n if n.startswith("t4") else "auto")
+        hd = 0 if n.startswith(("fast3d", "t4")) else (1 if n.startswith("stream3d") else -1)
         ok = run_case(kind, shape, T, dt, h, w0, ex, hd)
         print(f"{n}: {'ok' if ok else 'MISMATCH'}", flush=True)
         if not ok:
