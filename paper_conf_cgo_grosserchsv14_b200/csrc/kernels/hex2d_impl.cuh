@@ -81,7 +81,8 @@ struct Kernel {
   static constexpr int Q = R + 2;            // register rows q = b + 1, b in [-1, R]
   static constexpr int NT = NW * 32;
   static constexpr int C = NT * V;           // super-chunk width (classical tile w1)
-  static constexpr int MINB = sizeof(T) == 8 ? 2 : 3;  // resident CTAs/SM the register budget targets
+  // resident CTAs/SM the register budget targets: 12 (fp32) / 8 (fp64) warps per SM
+  static constexpr int MINB = (sizeof(T) == 8 ? 8 : 12) / NW > 0 ? (sizeof(T) == 8 ? 8 : 12) / NW : 1;
   static constexpr int NIN = W0 + 4 * H + 5; // In rows per chunk (= In values per column)
   static constexpr int SW = C + 8;           // staged row width (elements), 16-B granular
 
