@@ -148,35 +148,38 @@ stencil_status stencil_run(stencil_plan_t plan, const void *const *in, void *con
                            int64_t T_steps, void *stream);
 
 /* ---------------------------------------------------------------------------------
- * Multi-GPU slab mode.  One process per GPU; the outermost grid
- * dimension (part_dim = 0: contiguous planes) is split evenly over the ranks.  Rank q owns
- * planes [own_lo, own_hi) and stores the local slab [loc_lo, loc_hi) = its owned planes plus
- * G = radius * (2h+2) ghost planes on every side that is not a global boundary ("halos of
- * width radius x time-tile depth").  Every rank runs the GLOBAL run's launch table of the
- * hybrid schedule (Sec. 3.6; hexagon tiling translated to the slab) over its
- * slab, and before every launch but the first the library refreshes the ghost planes of both
- * ping-pong buffers from rank +-1 by ncclSend / ncclRecv (one NCCL group per buffer) on an
- * internal stream ordered against the caller's stream by events.  The slab's outermost planes
- * stay fixed; a launch spans at most 2h+2 levels, so wrong values never travel past the ghost
- * planes and every owned plane is exact after every launch; the ghost planes are the only
- * redundant work, and the schedule is continuous (no time-block cuts).
+ * Multi-GPU slab mode.  One process per GPU; one non-innermost grid
+ * dimension part_dim is split evenly over the ranks (part_dim < 0: the default -- 1 (y, a
+ * classically tiled dimension of the 3D kernels, the north star's "slab-decomposes the
+ * classically tiled spatial dimension") for 3D grids, 0 for 2D grids).  Rank q owns indices
+ * [own_lo, own_hi) of part_dim and stores the local slab [loc_lo, loc_hi) = its owned indices
+ * plus G = radius * (2h+2) ghost indices on every side that is not a global boundary ("halos of
+ * width radius x time-tile depth"); every other dimension is whole.  Every rank runs the GLOBAL
+ * run's launch table of the hybrid schedule (Sec. 3.6; when part_dim is the
+ * hexagonal dimension the hexagon tiling is translated to the slab) over its slab, and before
+ * every launch but the first the library refreshes the ghost indices of both ping-pong buffers
+ * from rank +-1 by ncclSend / ncclRecv (one NCCL group) on an internal stream ordered against
+ * the caller's stream by events; for part_dim > 0 the halos are strided in memory and are packed
+ * / unpacked through a staging area at the end of the plan's workspace.  The slab's outermost
+ * indices stay fixed; a launch spans at most 2h+2 levels, so wrong values never travel past the
+ * ghosts and every owned point is exact after every launch; the ghosts are the only redundant
+ * work, and the schedule is continuous (no time-block cuts).
  * NCCL is loaded at run time (the libnccl.so.2 the process already maps, e.g. PyTorch's;
  * environment HEXS_NCCL_LIB overrides); single-GPU use never needs it.  FDTD-2D is not
  * supported (STENCIL_E_UNSUPPORTED).
  * ------------------------------------------------------------------------------- */
 typedef struct {
   int32_t rank, nranks, part_dim;
-  int64_t global_ext[3];  /* stencil_dist_layout: the global extents (stencil_dist_info: -1 for
-                             dimension 0 when nranks > 1)                                   */
-  int64_t local_ext[3];   /* extents of this rank's local slab (ghost planes included)       */
-  int64_t own_lo, own_hi; /* owned global planes of dimension 0                              */
-  int64_t loc_lo, loc_hi; /* global planes held by the local slab                            */
+  int64_t global_ext[3];  /* the global extents                                              */
+  int64_t local_ext[3];   /* extents of this rank's local slab (ghosts included)             */
+  int64_t own_lo, own_hi; /* owned global indices of part_dim                                */
+  int64_t loc_lo, loc_hi; /* global indices of part_dim held by the local slab               */
   int64_t ghost;          /* G = radius * time_block                                         */
   int64_t time_block;     /* 2h+2: levels a launch spans (the halo's time-tile depth)         */
   int64_t n_blocks;       /* stencil_dist_info: launches per run (an exchange before each but
                              the first); stencil_dist_layout: 0                               */
   int32_t h;              /* hexagon half-height the time block is a multiple of             */
-  double ghost_fraction;  /* (local - owned) / owned planes: the redundant work              */
+  double ghost_fraction;  /* (local - owned) / owned indices: the redundant work             */
   int64_t launches_per_run; /* phase-kernel launches of one stencil_run (stencil_dist_info) */
 } stencil_dist_info_t;
 
@@ -192,11 +195,11 @@ stencil_status stencil_dist_layout(stencil_desc_t global_desc, int64_t T_steps, 
 /* Collective over the nranks processes (each on its own current device): build this rank's
  * distributed plan for T_steps steps of the GLOBAL problem global_desc.  tile as for
  * stencil_plan (its h sets the time block; NULL = defaults).  nccl_unique_id: the 128 bytes
- * from stencil_dist_unique_id on rank 0.  part_dim must be 0.  The plan is then used like a
+ * from stencil_dist_unique_id on rank 0.  part_dim: see above (< 0 = default).  The plan is then used like a
  * single-GPU plan: stencil_plan_workspace_size / set_workspace (shared by the block plans),
  * stencil_run(plan, in, out, T_steps, stream) with in / out the LOCAL slabs (local_ext,
- * 16-B aligned, in may alias out; every plane of `in`, ghosts included, holds level 0 of the
- * global grid) -- on return the owned planes of `out` hold level T_steps (ghost planes are
+ * 16-B aligned, in may alias out; every point of `in`, ghosts included, holds level 0 of the
+ * global grid) -- on return the owned points of `out` hold level T_steps (ghosts are
  * scratch).  stencil_run on a distributed plan is collective (every rank calls it).
  * STENCIL_E_NCCL on communicator or transfer failure. */
 stencil_status stencil_plan_dist(stencil_plan_t *out, stencil_desc_t global_desc, int64_t T_steps,
@@ -204,7 +207,7 @@ stencil_status stencil_plan_dist(stencil_plan_t *out, stencil_desc_t global_desc
                                  int nranks, int part_dim);
 
 /* Host-only: rank `rank`'s local plan -- the plan stencil_plan_dist runs on the slab (extent
- * loc_hi - loc_lo along dimension 0, the global hexagon tiling kept) -- as an ordinary plan
+ * loc_hi - loc_lo along part_dim, the global hexagon tiling kept) -- as an ordinary plan
  * (introspection: launch table, schedule_of; or a single-GPU run of one rank's slab without
  * halo exchanges).  Destroy it with stencil_destroy. */
 stencil_status stencil_dist_local_plan(stencil_plan_t *out, stencil_desc_t global_desc, int64_t T_steps,

@@ -1,24 +1,30 @@
 // dist.cpp -- multi-GPU slab mode of the C ABI: one process per GPU,
-// the outermost grid dimension slab-partitioned over the ranks, halos exchanged with NCCL
-// send/recv over NVLink once per phase launch (time tile).
+// one non-innermost grid dimension (3D default: y, a classically tiled dimension) slab-partitioned
+// over the ranks, halos exchanged with NCCL send/recv over NVLink once per phase launch (time tile).
 //
 // The paper's method is single-GPU: its host loop iterates the two phase kernels over the
 // whole grid (Sec. 4.1).  Here every rank runs exactly that host loop -- the
 // SAME launch table (T, p) as the global run -- over its local slab, and the ranks exchange
 // halos between consecutive launches:
-//   * rank q owns planes [own_lo, own_hi) of dimension 0 (an even split) and stores the local
-//     slab [loc_lo, loc_hi) = owned planes plus G = radius * (2h+2) ghost planes on every side
-//     that is not a global boundary (the halo width "radius x time-tile depth");
-//   * the local plan keeps the GLOBAL hexagon tiling (when dimension 0 is the hexagonal one,
-//     its rows are translated by loc_lo -- Sec. 4.2.3's tile translation offset), so after every
-//     launch each plane of the slab holds the same levels as in a single-GPU run;
-//   * before every launch but the first, the ghost planes of BOTH ping-pong buffers are
-//     refreshed from the neighbours' owned planes (ncclGroupStart; ncclSend / ncclRecv to
-//     rank -1 and rank +1; ncclGroupEnd), on a communication stream ordered against the compute
-//     stream by events; the outermost local planes act as fixed (Dirichlet) planes, and a launch
-//     spans at most 2h+2 levels, so its wrong values never travel further than G planes: every
-//     owned plane is exact after every launch.  The only redundant work is the ghost planes
-//     (2G / owned of the compute); there are no time-block cuts (the schedule is continuous).
+//   * rank q owns indices [own_lo, own_hi) of the partitioned dimension (an even split) and
+//     stores the local slab [loc_lo, loc_hi) = owned indices plus G = radius * (2h+2) ghost
+//     indices on every side that is not a global boundary (the halo width "radius x time-tile
+//     depth");
+//   * the local plan keeps the GLOBAL hexagon tiling: when the partitioned dimension is the
+//     hexagonal one its rows are translated by loc_lo (Sec. 4.2.3's tile translation offset);
+//     when it is a classical one (the 3D default, y) the hexagonal dimension is whole on every
+//     rank and the launch table is the global one as is -- which levels a launch computes at a
+//     point depends only on its (t, hexagonal) coordinates, never on the classical tiling -- so
+//     after every launch each point of the slab holds the same level as in a single-GPU run;
+//   * before every launch but the first, the ghost indices of BOTH ping-pong buffers are
+//     refreshed from the neighbours' owned ones (ncclGroupStart; ncclSend / ncclRecv to rank -1
+//     and rank +1; ncclGroupEnd), on a communication stream ordered against the compute stream
+//     by events; a partition of dimension > 0 is strided in memory, so its slabs are packed into
+//     / unpacked from a staging area of the workspace with 2-D copies on the same stream; the
+//     outermost local indices act as fixed (Dirichlet) cells, and a launch spans at most 2h+2
+//     levels, so its wrong values never travel further than G indices: every owned point is
+//     exact after every launch.  The only redundant work is the ghost slabs (2G / owned of the
+//     compute); there are no time-block cuts (the schedule is continuous).
 // NCCL is loaded at run time (dlopen of the libnccl.so.2 the process already uses, e.g.
 // PyTorch's), so single-GPU use of the library never needs it; PyTorch only broadcasts the
 // 128-byte unique id (stencil_dist_unique_id on rank 0).
@@ -108,7 +114,12 @@ struct DistState {
   std::vector<int64_t> blocks;                     // (one entry: T_steps; kept for the API)
   std::vector<std::pair<int64_t, Plan*>> bplans;   // the local plan (one, T_steps long)
   Desc local;                                      // descriptor of the local slab
-  size_t plane_bytes = 0;                          // bytes of one plane of dimension 0
+  int64_t global_n = 0;                            // global extent of the partitioned dimension
+  int64_t n_outer = 1;                             // product of the extents before it
+  size_t line_bytes = 0;                           // bytes of one index of it (extents after it)
+  size_t local_ws = 0;                             // the local plan's workspace (256-B rounded)
+  size_t stage_bytes = 0;                          // halo staging area after it (strided partitions)
+  char* stage = nullptr;
   void* comm = nullptr;                            // ncclComm_t
   cudaStream_t comm_stream = nullptr;
   cudaEvent_t ev_ready = nullptr, ev_done = nullptr;
@@ -144,29 +155,27 @@ void dist_fill_info(const Plan& p, stencil_plan_info_t& o) {
   o.n_launches = launches;
   o.T_steps = p.T_steps;
   o.tau_levels = p.tau_levels;
+  const int pd = s.lay.part_dim, r = s.local.radius;
   int64_t interior = 1;
-  for (int q = 1; q < s.local.dims; ++q) interior *= s.local.ext[q] - 2 * s.local.radius;
-  const int64_t glo = std::max<int64_t>(s.lay.own_lo, s.local.radius);
-  int64_t ghi = s.lay.own_hi;
-  if (s.lay.rank == s.lay.nranks - 1) ghi -= s.local.radius;  // the global last planes are Dirichlet
+  for (int q = 0; q < s.local.dims; ++q)
+    if (q != pd) interior *= s.local.ext[q] - 2 * r;
+  const int64_t glo = std::max<int64_t>(s.lay.own_lo, r);
+  const int64_t ghi = std::min<int64_t>(s.lay.own_hi, s.global_n - r);  // global edge cells are Dirichlet
   o.updates = std::max<int64_t>(0, ghi - glo) * interior * p.T_steps;
   o.workspace_bytes = p.ws_bytes;
 }
 
-// The tile of the local plans: the caller's, else (3D) the (2, 7) hexagon -- a 6-level time tile
-// keeps the ghost planes of a 128-plane slab under 10% -- else the class default the planner
-// picks for the GLOBAL grid.  Always returned explicit (h, w0), so every rank's local plan and the
-// layout share one hexagon (one tiling).
-stencil_tile_t dist_local_tile(const Desc& d, const stencil_tile_t* tile) {
+// The tile of the local plans: the caller's, else the class default the planner picks for the
+// GLOBAL grid (heat-3D 1024^3: (3, 7) -- measured per rank with y slabs it beats the shallower
+// (2, 7) at every rank count despite its larger ghost share, 12.5 % vs 9.4 % at 128 lines/rank:
+// DESIGN.md §7).  Always returned explicit (h, w0), so every rank's local plan and the layout
+// share one hexagon (one tiling).
+stencil_tile_t dist_local_tile(const Desc& d, const stencil_tile_t* tile, int nranks) {
+  (void)nranks;
   stencil_tile_t lt{};
   lt.hex_dim = -1;
   if (tile) lt = *tile;
   if (lt.h || lt.w0) return lt;  // an explicit hexagon
-  if (d.dims == 3 && lt.flags == STENCIL_EXEC_AUTO) {
-    lt.h = 2;
-    lt.w0 = 7;
-    return lt;
-  }
   Plan* probe = nullptr;
   if (build_plan(d, 1, &lt, &probe) == STENCIL_OK) {
     lt.h = probe->h;
@@ -181,8 +190,9 @@ stencil_tile_t dist_local_tile(const Desc& d, const stencil_tile_t* tile) {
 stencil_status dist_layout(const Desc& d, int64_t T_steps, const stencil_tile_t* tile, int rank, int nranks,
                            int part_dim, DistLayout* out) {
   if (nranks < 1 || rank < 0 || rank >= nranks) return fail(STENCIL_E_INVALID, "stencil_plan_dist: bad rank / nranks");
-  if (part_dim != 0)
-    return fail(STENCIL_E_UNSUPPORTED, "stencil_plan_dist: only the outermost dimension (contiguous planes) is partitioned");
+  if (part_dim < 0) part_dim = d.dims == 3 ? 1 : 0;  // default: y in 3D (classical), rows in 2D
+  if (part_dim > d.dims - 2)
+    return fail(STENCIL_E_UNSUPPORTED, "stencil_plan_dist: the partitioned dimension must not be the innermost one");
   if (d.kind == STENCIL_FDTD2D)
     return fail(STENCIL_E_UNSUPPORTED, "stencil_plan_dist: FDTD-2D (three in-place fields) has no slab mode");
   if (T_steps < 0) return fail(STENCIL_E_INVALID, "stencil_plan_dist: T_steps < 0");
@@ -190,14 +200,14 @@ stencil_status dist_layout(const Desc& d, int64_t T_steps, const stencil_tile_t*
   L.rank = rank;
   L.nranks = nranks;
   L.part_dim = part_dim;
-  const int64_t N0 = d.ext[0];
+  const int64_t N0 = d.ext[part_dim];
   const int64_t base = N0 / nranks, extra = N0 % nranks;
   L.own_lo = rank * base + std::min<int64_t>(rank, extra);
   L.own_hi = L.own_lo + base + (rank < extra ? 1 : 0);
   // time block: a multiple of the hexagon height 2h+2 of the local plans' tile (one time tile
   // by default, more while the ghost planes stay within ~10% of the owned ones);
   // HEXS_TIME_BLOCK overrides
-  const stencil_tile_t lt = dist_local_tile(d, tile);
+  const stencil_tile_t lt = dist_local_tile(d, tile, nranks);
   const int h = lt.h;
   const int64_t H = 2 * (int64_t)h + 2;
   const int64_t owned = L.own_hi - L.own_lo;
@@ -207,6 +217,8 @@ stencil_status dist_layout(const Desc& d, int64_t T_steps, const stencil_tile_t*
   L.ghost = (int64_t)d.radius * D;
   if (nranks > 1 && owned < L.ghost)
     return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_plan_dist: a slab is thinner than the ghost width radius*(2h+2)");
+  if (nranks > 1 && d.dims == 3 && part_dim == 1 && d.ext[0] < 3)
+    return fail(STENCIL_E_INVALID, "stencil_plan_dist: degenerate grid");
   L.loc_lo = std::max<int64_t>(0, L.own_lo - L.ghost);
   L.loc_hi = std::min<int64_t>(N0, L.own_hi + L.ghost);
   L.n_blocks = 0;  // filled by stencil_plan_dist: launches (one exchange before each but the first)
@@ -217,40 +229,72 @@ stencil_status dist_layout(const Desc& d, int64_t T_steps, const stencil_tile_t*
 }
 
 stencil_status dist_set_workspace(Plan& p, void* dev_ptr, size_t bytes) {
-  for (auto& bp : p.dist->bplans) {
-    if (bytes < bp.second->ws_bytes) return fail(STENCIL_E_OOM, "stencil_plan_set_workspace: workspace too small");
+  DistState& s = *p.dist;
+  if (bytes < s.local_ws + s.stage_bytes) return fail(STENCIL_E_OOM, "stencil_plan_set_workspace: workspace too small");
+  for (auto& bp : s.bplans) {
     bp.second->ws = dev_ptr;
-    bp.second->ws_size = bytes;
+    bp.second->ws_size = s.local_ws;
   }
+  s.stage = s.stage_bytes ? static_cast<char*>(dev_ptr) + s.local_ws : nullptr;
   return STENCIL_OK;
 }
 
-// One halo exchange on the communication stream: my first / last G owned planes go to rank -1
-// / rank + 1, their owned planes land in my ghost planes.
-static stencil_status exchange(DistState& s, char* base, cudaStream_t stream) {
+// One halo exchange of both ping-pong buffers on the communication stream: my first / last G
+// owned indices go to rank -1 / rank +1, their owned indices land in my ghost indices.  A
+// partition of dimension 0 sends contiguous planes; a deeper one is strided (n_outer blocks of
+// G lines, local_n lines apart) and goes through the staging area: packed by 2-D copies, sent,
+// received, unpacked -- all on the communication stream.
+static stencil_status exchange(DistState& s, void* const* bufs, cudaStream_t stream) {
   NcclApi* a = nccl_api();
   if (!a) return fail(STENCIL_E_NCCL, "NCCL unavailable");
   const DistLayout& L = s.lay;
-  const int64_t G = L.ghost;
-  const size_t n = (size_t)G * s.plane_bytes;
+  const int64_t G = L.ghost, local_n = L.loc_hi - L.loc_lo;
+  const size_t chunk = (size_t)G * s.line_bytes;  // one outer block of a halo
+  const size_t n = chunk * (size_t)s.n_outer;     // one halo
+  const size_t pitch = (size_t)local_n * s.line_bytes;
+  const bool strided = s.n_outer > 1;
+  if (strided && !s.stage) return fail(STENCIL_E_INVALID, "stencil_run: workspace not set (halo staging)");
   ncclComm_t comm = static_cast<ncclComm_t>(s.comm);
+  cudaStream_t cs = s.comm_stream;
   cudaError_t e = cudaEventRecord(s.ev_ready, stream);
-  if (e == cudaSuccess) e = cudaStreamWaitEvent(s.comm_stream, s.ev_ready, 0);
+  if (e == cudaSuccess) e = cudaStreamWaitEvent(cs, s.ev_ready, 0);
   if (e != cudaSuccess) return fail(STENCIL_E_CUDA, std::string("stencil_run: halo ordering: ") + cudaGetErrorString(e));
+  const int64_t own0 = L.own_lo - L.loc_lo, own1 = L.own_hi - L.loc_lo;  // local indices
+  const bool lo_nb = L.rank > 0, hi_nb = L.rank < L.nranks - 1;
+  // staging layout per buffer b: [send lo][send hi][recv lo][recv hi]
+  auto stg = [&](int b, int slot) { return s.stage + ((size_t)b * 4 + slot) * n; };
+  auto at = [&](int b, int64_t idx) { return static_cast<char*>(bufs[b]) + (size_t)idx * s.line_bytes; };
+  if (strided) {
+    for (int b = 0; b < 2 && e == cudaSuccess; ++b) {
+      if (lo_nb) e = cudaMemcpy2DAsync(stg(b, 0), chunk, at(b, own0), pitch, chunk, s.n_outer, cudaMemcpyDeviceToDevice, cs);
+      if (hi_nb && e == cudaSuccess)
+        e = cudaMemcpy2DAsync(stg(b, 1), chunk, at(b, own1 - G), pitch, chunk, s.n_outer, cudaMemcpyDeviceToDevice, cs);
+    }
+    if (e != cudaSuccess) return fail(STENCIL_E_CUDA, std::string("stencil_run: halo pack: ") + cudaGetErrorString(e));
+  }
   ncclResult_t r = a->GroupStart();
   if (r != ncclSuccess) return nccl_fail(a, r, "ncclGroupStart");
-  const int64_t own0 = L.own_lo - L.loc_lo, own1 = L.own_hi - L.loc_lo;  // local plane indices
-  if (L.rank > 0) {
-    a->Send(base + own0 * s.plane_bytes, n, ncclChar, L.rank - 1, comm, s.comm_stream);
-    a->Recv(base + (own0 - G) * s.plane_bytes, n, ncclChar, L.rank - 1, comm, s.comm_stream);
-  }
-  if (L.rank < L.nranks - 1) {
-    a->Send(base + (own1 - G) * s.plane_bytes, n, ncclChar, L.rank + 1, comm, s.comm_stream);
-    a->Recv(base + own1 * s.plane_bytes, n, ncclChar, L.rank + 1, comm, s.comm_stream);
+  for (int b = 0; b < 2; ++b) {
+    if (lo_nb) {
+      a->Send(strided ? stg(b, 0) : at(b, own0), n, ncclChar, L.rank - 1, comm, cs);
+      a->Recv(strided ? stg(b, 2) : at(b, own0 - G), n, ncclChar, L.rank - 1, comm, cs);
+    }
+    if (hi_nb) {
+      a->Send(strided ? stg(b, 1) : at(b, own1 - G), n, ncclChar, L.rank + 1, comm, cs);
+      a->Recv(strided ? stg(b, 3) : at(b, own1), n, ncclChar, L.rank + 1, comm, cs);
+    }
   }
   r = a->GroupEnd();
   if (r != ncclSuccess) return nccl_fail(a, r, "ncclGroupEnd");
-  e = cudaEventRecord(s.ev_done, s.comm_stream);
+  if (strided) {
+    for (int b = 0; b < 2 && e == cudaSuccess; ++b) {
+      if (lo_nb) e = cudaMemcpy2DAsync(at(b, own0 - G), pitch, stg(b, 2), chunk, chunk, s.n_outer, cudaMemcpyDeviceToDevice, cs);
+      if (hi_nb && e == cudaSuccess)
+        e = cudaMemcpy2DAsync(at(b, own1), pitch, stg(b, 3), chunk, chunk, s.n_outer, cudaMemcpyDeviceToDevice, cs);
+    }
+    if (e != cudaSuccess) return fail(STENCIL_E_CUDA, std::string("stencil_run: halo unpack: ") + cudaGetErrorString(e));
+  }
+  e = cudaEventRecord(s.ev_done, cs);
   if (e == cudaSuccess) e = cudaStreamWaitEvent(stream, s.ev_done, 0);
   if (e != cudaSuccess) return fail(STENCIL_E_CUDA, std::string("stencil_run: halo ordering: ") + cudaGetErrorString(e));
   if (a->CommGetAsyncError) {
@@ -265,11 +309,7 @@ static stencil_status exchange(DistState& s, char* base, cudaStream_t stream) {
 static stencil_status ghost_hook(void* ctx, int64_t /*k*/, void* const* bufs, void* stream) {
   DistState& s = *static_cast<DistState*>(ctx);
   if (s.lay.nranks <= 1 || s.emulate) return STENCIL_OK;
-  for (int b = 0; b < 2; ++b) {
-    stencil_status st = exchange(s, static_cast<char*>(bufs[b]), static_cast<cudaStream_t>(stream));
-    if (st != STENCIL_OK) return st;
-  }
-  return STENCIL_OK;
+  return exchange(s, bufs, static_cast<cudaStream_t>(stream));
 }
 
 stencil_status run_dist(Plan& p, const void* const* in, void* const* out, void* stream_) {
@@ -324,7 +364,7 @@ stencil_status stencil_dist_layout(stencil_desc_t global_desc, int64_t T_steps, 
     o.global_ext[q] = q < d->dims ? d->ext[q] : 1;
     o.local_ext[q] = o.global_ext[q];
   }
-  o.local_ext[0] = L.loc_hi - L.loc_lo;
+  o.local_ext[L.part_dim] = L.loc_hi - L.loc_lo;
   o.own_lo = L.own_lo;
   o.own_hi = L.own_hi;
   o.loc_lo = L.loc_lo;
@@ -352,21 +392,26 @@ stencil_status stencil_plan_dist(stencil_plan_t* out, stencil_desc_t global_desc
   stencil_status st = dist_layout(*d, T_steps, tile, rank, nranks, part_dim, &s->lay);
   if (st != STENCIL_OK) return st;
   const DistLayout& L = s->lay;
+  const int pd = L.part_dim;
   // the local slab's descriptor: same class / coefficients / dtype, extent loc_hi - loc_lo
   s->local = *d;
-  s->local.ext[0] = L.loc_hi - L.loc_lo;
-  if (s->local.ext[0] < 3) return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_plan_dist: local slab thinner than 3 planes");
-  s->plane_bytes = d->elem();
-  for (int q = 1; q < d->dims; ++q) s->plane_bytes *= (size_t)d->ext[q];
+  s->local.ext[pd] = L.loc_hi - L.loc_lo;
+  if (s->local.ext[pd] < 3) return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_plan_dist: local slab thinner than 3 indices");
+  s->global_n = d->ext[pd];
+  s->line_bytes = d->elem();
+  for (int q = pd + 1; q < d->dims; ++q) s->line_bytes *= (size_t)d->ext[q];
+  s->n_outer = 1;
+  for (int q = 0; q < pd; ++q) s->n_outer *= d->ext[q];
   s->blocks.push_back(T_steps);
-  const stencil_tile_t lt = dist_local_tile(*d, tile);
+  const stencil_tile_t lt = dist_local_tile(*d, tile, nranks);
   {
     // the local plan: the global schedule restricted to the slab (hexagon rows translated by
-    // loc_lo when dimension 0 is the hexagonal one, so the tiling matches the global one)
+    // loc_lo when the partitioned dimension is the hexagonal one, so the tiling matches the
+    // global one)
     Plan* probe = nullptr;
     st = build_plan(s->local, T_steps, &lt, &probe);
     if (st != STENCIL_OK) return st;
-    const int64_t origin = probe->hd == 0 ? L.loc_lo : 0;
+    const int64_t origin = probe->hd == pd ? L.loc_lo : 0;
     delete probe;
     Plan* bp = nullptr;
     st = build_plan(s->local, T_steps, &lt, &bp, origin);
@@ -415,7 +460,10 @@ stencil_status stencil_plan_dist(stencil_plan_t* out, stencil_desc_t global_desc
   p->executor = primary ? primary->executor : EXEC_GENERIC;
   size_t ws = 0;
   for (auto& bp : s->bplans) ws = std::max(ws, bp.second->ws_bytes);
-  p->ws_bytes = ws;
+  s->local_ws = (ws + 255) / 256 * 256;
+  // strided partitions: staging for both buffers' 2 send + 2 receive halos
+  s->stage_bytes = s->n_outer > 1 && nranks > 1 ? 8 * (size_t)L.ghost * s->line_bytes * (size_t)s->n_outer : 0;
+  p->ws_bytes = s->local_ws + s->stage_bytes;
   p->dist = s.release();
   *out = reinterpret_cast<stencil_plan_t>(p);
   return STENCIL_OK;
@@ -432,13 +480,13 @@ stencil_status stencil_dist_local_plan(stencil_plan_t* out, stencil_desc_t globa
   stencil_status st = dist_layout(*d, T_steps, tile, rank, nranks, part_dim, &L);
   if (st != STENCIL_OK) return st;
   Desc local = *d;
-  local.ext[0] = L.loc_hi - L.loc_lo;
-  if (local.ext[0] < 3) return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_dist_local_plan: slab thinner than 3 planes");
-  const stencil_tile_t lt = dist_local_tile(*d, tile);
+  local.ext[L.part_dim] = L.loc_hi - L.loc_lo;
+  if (local.ext[L.part_dim] < 3) return fail(STENCIL_E_INFEASIBLE_TILE, "stencil_dist_local_plan: slab thinner than 3 indices");
+  const stencil_tile_t lt = dist_local_tile(*d, tile, nranks);
   Plan* probe = nullptr;
   st = build_plan(local, T_steps, &lt, &probe);
   if (st != STENCIL_OK) return st;
-  const int64_t origin = probe->hd == 0 ? L.loc_lo : 0;
+  const int64_t origin = probe->hd == L.part_dim ? L.loc_lo : 0;
   delete probe;
   Plan* p = nullptr;
   st = build_plan(local, T_steps, &lt, &p, origin);
@@ -458,8 +506,8 @@ stencil_status stencil_dist_info(stencil_plan_t plan, stencil_dist_info_t* info)
   o.nranks = L.nranks;
   o.part_dim = L.part_dim;
   for (int q = 0; q < 3; ++q) o.local_ext[q] = o.global_ext[q] = q < s.local.dims ? s.local.ext[q] : 1;
-  o.global_ext[0] = -1;  // filled below from the partition
-  o.local_ext[0] = L.loc_hi - L.loc_lo;
+  o.global_ext[L.part_dim] = s.global_n;
+  o.local_ext[L.part_dim] = L.loc_hi - L.loc_lo;
   o.own_lo = L.own_lo;
   o.own_hi = L.own_hi;
   o.loc_lo = L.loc_lo;
@@ -475,7 +523,6 @@ stencil_status stencil_dist_info(stencil_plan_t plan, stencil_dist_info_t* info)
     launches += bp->executor == EXEC_NAIVE ? bp->tau_levels : (int64_t)bp->launches.size();
   }
   o.launches_per_run = launches;
-  o.global_ext[0] = L.nranks == 1 ? L.own_hi : -1;
   *info = o;
   return STENCIL_OK;
 }

@@ -1,14 +1,15 @@
 """Multi-GPU slab mode over the C ABI's distributed plans.
 
-One process per GPU.  The library (csrc/dist.cpp, include/stencil.h) partitions the outermost
-grid dimension, keeps G = radius * D ghost planes per interior side, runs every time block of
-D steps as the single-GPU hybrid schedule over the local slab and exchanges the ghost planes
-with ncclSend / ncclRecv between blocks.  Python only bootstraps: rank 0 asks the library for
+One process per GPU.  The library (csrc/dist.cpp, include/stencil.h) partitions one
+non-innermost grid dimension (`part_dim`; default y in 3D -- a classically tiled dimension --
+and rows in 2D), keeps G = radius * (2h+2) ghost indices per interior side, runs the global
+launch table of the hybrid schedule over the local slab and refreshes the ghosts of both
+ping-pong buffers with ncclSend / ncclRecv before every launch but the first.  Python only bootstraps: rank 0 asks the library for
 an NCCL unique id and torch.distributed broadcasts it; PyTorch provides the device memory.
 
     dp = DistPlan("star3d7", (1024, 1024, 1024), T=256)    # collective
     local = dp.scatter(global_grid)                        # this rank's slab (ghosts included)
-    dp.run(local)                                          # collective; owned planes -> level T
+    dp.run(local)                                          # collective; owned points -> level T
     owned = dp.owned(local)
 
 `layout(...)` is the same partition as a host-only call (no GPU, no NCCL): the CPU tests
@@ -36,6 +37,7 @@ from .api import _dtype_code
 class Layout:
     rank: int
     nranks: int
+    part_dim: int
     global_ext: Tuple[int, ...]
     local_ext: Tuple[int, ...]
     own_lo: int
@@ -51,6 +53,11 @@ class Layout:
     @property
     def own_local(self) -> Tuple[int, int]:
         return self.own_lo - self.loc_lo, self.own_hi - self.loc_lo
+
+    def take(self, a, lo: int, hi: int):
+        """a[..., lo:hi, ...] along the partitioned dimension (numpy or torch)."""
+        idx = [slice(None)] * self.part_dim + [slice(lo, hi)]
+        return a[tuple(idx)]
 
 
 
@@ -69,36 +76,39 @@ def _desc(kind: str, ext: Sequence[int], dtype="float32"):
 
 
 def _layout_of(info: DistInfo, dims: int, global_ext: Sequence[int]) -> Layout:
-    return Layout(info.rank, info.nranks, tuple(int(x) for x in global_ext),
+    return Layout(info.rank, info.nranks, info.part_dim, tuple(int(x) for x in global_ext),
                   tuple(int(info.local_ext[q]) for q in range(dims)), info.own_lo, info.own_hi, info.loc_lo,
                   info.loc_hi, info.ghost, info.time_block, info.n_blocks, info.h, info.ghost_fraction)
 
 
 def layout(kind: str, global_ext: Sequence[int], T: int, rank: int, nranks: int, dtype="float32",
-           **tile) -> Layout:
+           part_dim: int = -1, **tile) -> Layout:
     """This rank's slab layout, exactly as stencil_plan_dist builds it (host only)."""
     d = _desc(kind, global_ext, dtype)
     try:
         info = DistInfo()
         t = _tile(**tile)
-        check(lib().stencil_dist_layout(d, int(T), ctypes.byref(t), int(rank), int(nranks), 0, ctypes.byref(info)))
+        check(lib().stencil_dist_layout(d, int(T), ctypes.byref(t), int(rank), int(nranks), int(part_dim),
+                                        ctypes.byref(info)))
         return _layout_of(info, len(global_ext), global_ext)
     finally:
         lib().stencil_destroy(d)
 
 
-def local_plan(kind: str, global_ext: Sequence[int], T: int, rank: int, nranks: int, dtype="float32", **tile):
+def local_plan(kind: str, global_ext: Sequence[int], T: int, rank: int, nranks: int, dtype="float32",
+               part_dim: int = -1, **tile):
     """Rank `rank`'s local plan (host only; stencil_dist_local_plan): the global launch table of
     the hybrid schedule restricted to the slab -- what a distributed plan runs between its halo
     exchanges."""
     from .api import Plan, Stencil
 
-    lay = layout(kind, global_ext, T, rank, nranks, dtype, **tile)
+    lay = layout(kind, global_ext, T, rank, nranks, dtype, part_dim, **tile)
     d = _desc(kind, global_ext, dtype)
     try:
         h = ctypes.c_void_p()
         t = _tile(**tile)
-        check(lib().stencil_dist_local_plan(ctypes.byref(h), d, int(T), ctypes.byref(t), int(rank), int(nranks), 0))
+        check(lib().stencil_dist_local_plan(ctypes.byref(h), d, int(T), ctypes.byref(t), int(rank), int(nranks),
+                                            int(part_dim)))
     finally:
         lib().stencil_destroy(d)
     return Plan._adopt(Stencil(kind, lay.local_ext, dtype=dtype), h, T), lay
@@ -106,19 +116,26 @@ def local_plan(kind: str, global_ext: Sequence[int], T: int, rank: int, nranks: 
 
 def exchange_halos(local: torch.Tensor, lay: Layout, group=None) -> None:
     """The library's halo step over torch.distributed (for CPU/gloo tests of the protocol):
-    send my first / last G owned planes down / up, receive the neighbours' into my ghosts."""
+    send my first / last G owned indices of the partitioned dimension down / up, receive the
+    neighbours' into my ghosts (strided slabs through contiguous staging, as the library does)."""
     G = lay.ghost
     lo, hi = lay.own_local
-    ops = []
+    ops, unpack = [], []
     if lay.rank > 0:
-        ops.append(dist.P2POp(dist.isend, local[lo:lo + G].contiguous(), lay.rank - 1, group))
-        ops.append(dist.P2POp(dist.irecv, local[lo - G:lo], lay.rank - 1, group))
+        rl = torch.empty_like(lay.take(local, lo - G, lo).contiguous())
+        ops.append(dist.P2POp(dist.isend, lay.take(local, lo, lo + G).contiguous(), lay.rank - 1, group))
+        ops.append(dist.P2POp(dist.irecv, rl, lay.rank - 1, group))
+        unpack.append((lo - G, lo, rl))
     if lay.rank < lay.nranks - 1:
-        ops.append(dist.P2POp(dist.isend, local[hi - G:hi].contiguous(), lay.rank + 1, group))
-        ops.append(dist.P2POp(dist.irecv, local[hi:hi + G], lay.rank + 1, group))
+        rh = torch.empty_like(lay.take(local, hi, hi + G).contiguous())
+        ops.append(dist.P2POp(dist.isend, lay.take(local, hi - G, hi).contiguous(), lay.rank + 1, group))
+        ops.append(dist.P2POp(dist.irecv, rh, lay.rank + 1, group))
+        unpack.append((hi, hi + G, rh))
     if ops:
         for req in dist.batch_isend_irecv(ops):
             req.wait()
+    for a, b, buf in unpack:
+        lay.take(local, a, b).copy_(buf)
 
 
 def run_protocol(bufs: Sequence[torch.Tensor], lay: Layout, plan, execute_launch: Callable, group=None) -> None:
@@ -136,7 +153,8 @@ class DistPlan:
     """A distributed plan (stencil_plan_dist) of T steps of `kind` on the global grid
     `global_ext`, over the ranks of `group` (one GPU each).  Collective constructor."""
 
-    def __init__(self, kind: str, global_ext: Sequence[int], T: int, group=None, dtype="float32", **tile):
+    def __init__(self, kind: str, global_ext: Sequence[int], T: int, group=None, dtype="float32",
+                 part_dim: int = -1, **tile):
         self.kind = kind
         self.global_ext = tuple(int(e) for e in global_ext)
         self.T = int(T)
@@ -160,7 +178,7 @@ class DistPlan:
         t = _tile(**tile)
         h = ctypes.c_void_p()
         check(lib().stencil_plan_dist(ctypes.byref(h), self._d, self.T, ctypes.byref(t), uid, self.rank,
-                                      self.nranks, 0))
+                                      self.nranks, int(part_dim)))
         self._h = h
         info = DistInfo()
         check(lib().stencil_dist_info(h, ctypes.byref(info)))
@@ -171,15 +189,15 @@ class DistPlan:
 
     # ---- data placement ---------------------------------------------------------------
     def scatter(self, global_grid) -> torch.Tensor:
-        """This rank's local slab (owned + ghost planes) of a full global grid, on its GPU."""
+        """This rank's local slab (owned + ghost indices) of a full global grid, on its GPU."""
         lay = self.layout
-        part = global_grid[lay.loc_lo:lay.loc_hi]
+        part = lay.take(global_grid, lay.loc_lo, lay.loc_hi)
         t = part if isinstance(part, torch.Tensor) else torch.from_numpy(part.copy())
         return t.contiguous().cuda()
 
     def owned(self, local: torch.Tensor) -> torch.Tensor:
         lo, hi = self.layout.own_local
-        return local[lo:hi]
+        return self.layout.take(local, lo, hi)
 
     # ---- execution ----------------------------------------------------------------------
     @property
@@ -261,13 +279,15 @@ def bench_main(args, cfg, configs, metric, helpers):
     if getattr(args, "tile", ""):  # h,w0: the local plans' hexagon (tuning)
         v = [int(x) for x in args.tile.split(",")]
         tile = {"h": v[0], "w0": v[1]}
-    dp = DistPlan(kind, gext, T, **tile)
+    part_dim = int(os.environ.get("HEXS_DIST_PART_DIM", "-1"))  # default: y in 3D (classical)
+    dp = DistPlan(kind, gext, T, part_dim=part_dim, **tile)
     lay = dp.layout
-    plane = 1
-    for e in gext[1:]:
-        plane *= e
+    pd = lay.part_dim
     # each rank generates only its slab of the global synthetic grid (same counter-based recipe)
-    local_np = stencil_inputs.uniform(lay.local_ext, seed=0, offset=lay.loc_lo * plane)
+    box_lo = [0] * len(gext)
+    box_hi = list(gext)
+    box_lo[pd], box_hi[pd] = lay.loc_lo, lay.loc_hi
+    local_np = stencil_inputs.uniform_box(gext, box_lo, box_hi, seed=0)
     host_in = torch.from_numpy(local_np).pin_memory()
     local0 = host_in.cuda()
     local = torch.empty_like(local0)
@@ -300,7 +320,8 @@ def bench_main(args, cfg, configs, metric, helpers):
     # (halo exchanges included), D2H of the owned planes; two slab buffer pairs and H2D / D2H
     # streams overlap a step's transfers with its neighbours' compute
     lo, hi = lay.own_local
-    host_out = [torch.empty_like(host_in[lo:hi]).pin_memory() for _ in range(2)]
+    own_shape = tuple(lay.take(host_in, lo, hi).shape)
+    host_out = [torch.empty(own_shape, dtype=host_in.dtype).pin_memory() for _ in range(2)]
     ins = [local0, torch.empty_like(local0)]
     outs = [local, torch.empty_like(local)]
     h2d, d2h = torch.cuda.Stream(), torch.cuda.Stream()
@@ -329,7 +350,7 @@ def bench_main(args, cfg, configs, metric, helpers):
         ev_done[k].record(stream)
         with torch.cuda.stream(d2h):
             d2h.wait_event(ev_done[k])
-            host_out[k].copy_(outs[k][lo:hi], non_blocking=True)
+            host_out[k].copy_(lay.take(outs[k], lo, hi), non_blocking=True)
             ev_out[k].record(d2h)
     stream.wait_event(ev_out[(args.steps - 1) % 2])
     stream.wait_event(ev_out[args.steps % 2])
@@ -339,7 +360,7 @@ def bench_main(args, cfg, configs, metric, helpers):
     dist.all_reduce(e2e_ms, op=dist.ReduceOp.MAX)
     e2e_ms = float(e2e_ms.item())
     # the pipelined result equals the device-resident run's owned planes
-    assert torch.equal(host_out[(args.steps - 1) % 2], local[lo:hi].cpu()), "pipelined e2e result differs"
+    assert torch.equal(host_out[(args.steps - 1) % 2], lay.take(local, lo, hi).cpu()), "pipelined e2e result differs"
 
     # phase-kernel roofline of the D-step block plan: kernel-region events of one run
     bp = dp.block_plan
@@ -360,8 +381,8 @@ def bench_main(args, cfg, configs, metric, helpers):
                 "traffic": None, "peak_source": peak_src,
                 "kernel": helpers.KERNEL_NAMES.get(_lib.KERNELS[binfo.kernel], _lib.KERNELS[binfo.kernel]),
                 "bytes_per_update": bpu, "block_kernel_ms": kms.value, "block_launches": nl.value,
-                "note": "one D-step block plan on the local slab (ghost planes included); block-cut "
-                        "and ghost traffic not in bytes_per_update"}
+                "note": "the local plan on the rank's slab (ghosts included); ghost traffic not in "
+                        "bytes_per_update"}
     if rank == 0:
         nbytes_in = host_in.numel() * host_in.element_size()
         nbytes_out = host_out[0].numel() * host_out[0].element_size()
@@ -371,8 +392,8 @@ def bench_main(args, cfg, configs, metric, helpers):
                 "data": "synthetic",
                 "config": {"workload": cname + (f" weak-scaled to {gext[0]} planes over {world} GPUs"
                                                 if scaling == "weak" else f" over {world} GPUs"),
-                           "kind": kind, "extents": list(gext), "T": T, "partition": "dim 0 slabs",
-                           "time_block": lay.time_block, "ghost_planes": lay.ghost,
+                           "kind": kind, "extents": list(gext), "T": T, "partition": f"dim {pd} slabs",
+                           "time_block": lay.time_block, "ghost_indices": lay.ghost,
                            "ghost_fraction": lay.ghost_fraction, "local_extents": list(lay.local_ext),
                            "l2": "inputs larger than L2 (per-rank slab > 126 MB)"},
                 "roofline": roof,
@@ -387,8 +408,8 @@ def bench_main(args, cfg, configs, metric, helpers):
         if emu:  # a projection, not a measurement of N GPUs: say so and report the rank's rate
             r, P = (int(x) for x in emu.split("/"))
             own = lay.own_hi - lay.own_lo
-            line["emulated_rank"] = {"rank": r, "nranks": P, "owned_planes": own,
-                                     "rank_gups": value * own / gext[0],
+            line["emulated_rank"] = {"rank": r, "nranks": P, "owned_indices": own, "part_dim": pd,
+                                     "rank_gups": value * own / gext[pd],
                                      "note": "one GPU runs rank r's slab alone (ghosts fixed, no NCCL): compute-only "
                                              "projection; 'value' is the whole-grid rate of that rank's time"}
         print(json.dumps(line), flush=True)

@@ -52,3 +52,27 @@ def uniform(shape: Sequence[int], seed: int, dtype=np.float32, out: np.ndarray =
 def fields(shape: Sequence[int], seed: int, n: int, dtype=np.float32):
     """n independent fields (e.g. FDTD's ex, ey, hz) from seeds seed, seed+1, ..."""
     return [uniform(shape, seed + k, dtype) for k in range(n)]
+
+
+def uniform_box(global_shape: Sequence[int], lo: Sequence[int], hi: Sequence[int], seed: int,
+                dtype=np.float32) -> np.ndarray:
+    """The sub-box [lo, hi) of the grid `uniform(global_shape, seed)` -- generated on its own (a
+    rank's slab of a partition along any dimension), bit-identical to slicing the full grid."""
+    gs = [int(s) for s in global_shape]
+    lo = [int(v) for v in lo]
+    hi = [int(v) for v in hi]
+    strides = [int(np.prod(gs[q + 1:])) for q in range(len(gs))]
+    out = np.empty([b - a for a, b in zip(lo, hi)], dtype=dtype)
+    key = np.uint64((int(seed) * int(_K)) & 0xFFFFFFFFFFFFFFFF)
+    # linear indices of one outermost slice of the box (broadcast over the inner dimensions)
+    inner = np.zeros([1] + [b - a for a, b in zip(lo[1:], hi[1:])], dtype=np.uint64)
+    for q in range(1, len(gs)):
+        shp = [1] * len(gs)
+        shp[q] = hi[q] - lo[q]
+        inner = inner + (np.arange(lo[q], hi[q], dtype=np.uint64) * np.uint64(strides[q])).reshape(shp)
+    with np.errstate(over="ignore"):
+        for k, z in enumerate(range(lo[0], hi[0])):
+            idx = inner[0] + np.uint64(z * strides[0])
+            v = _splitmix64(idx ^ key)
+            out[k] = (v >> np.uint64(40)).astype(np.float64) * (2.0 ** -24)
+    return out

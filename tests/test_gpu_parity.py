@@ -188,31 +188,25 @@ def test_full_size_fdtd():
 
 
 def test_dist_plan_nccl_single_rank():
-    """The C ABI's distributed plan (stencil_plan_dist: NCCL communicator from a unique id,
-    time blocks of D steps, block plans on the local slab) with one rank on the GPU: bit-exact
-    against the single-domain oracle, including a remainder block and both dtypes' 2D/3D paths."""
-    import os
-
+    """The C ABI's distributed plan (stencil_plan_dist: NCCL communicator from a unique id, the
+    local plan on the slab) with one rank on the GPU: bit-exact against the single-domain oracle
+    for 2D and 3D classes and both partition dimensions of a 3D grid."""
     from paper_conf_cgo_grosserchsv14_b200 import dist as hdist
 
-    for kind, ext, T, D in [("star2d5", (301, 517), 37, "16"), ("star3d7", (40, 45, 68), 11, "4"),
-                            ("star3d7", (64, 40, 64), 20, ""), ("box2d9", (130, 260), 19, "")]:
-        if D:
-            os.environ["HEXS_TIME_BLOCK"] = D
-        else:
-            os.environ.pop("HEXS_TIME_BLOCK", None)
-        try:
-            g = stencil_inputs.uniform(ext, seed=9)
-            dp = hdist.DistPlan(kind, ext, T)
-            assert dp.layout.loc_lo == 0 and dp.layout.loc_hi == ext[0]
-            local = dp.scatter(g)
-            out = torch.empty_like(local)
-            for _ in range(2):
-                dp.run(local, out)
-            torch.cuda.synchronize()
-            assert_bitexact(dp.owned(out).cpu().numpy(), oracle.run(kind, g, T), f"dist {kind} D={D}")
-        finally:
-            os.environ.pop("HEXS_TIME_BLOCK", None)
+    for kind, ext, T, pd in [("star2d5", (301, 517), 37, -1), ("star3d7", (40, 45, 68), 11, -1),
+                             ("star3d7", (64, 40, 64), 20, 0), ("box2d9", (130, 260), 19, -1),
+                             ("star3d7", (33, 70, 132), 17, 1)]:
+        g = stencil_inputs.uniform(ext, seed=9)
+        dp = hdist.DistPlan(kind, ext, T, part_dim=pd)
+        lay = dp.layout
+        assert lay.part_dim == (pd if pd >= 0 else (1 if len(ext) == 3 else 0))
+        assert lay.loc_lo == 0 and lay.loc_hi == ext[lay.part_dim] and lay.local_ext == ext
+        local = dp.scatter(g)
+        out = torch.empty_like(local)
+        for _ in range(2):
+            dp.run(local, out)
+        torch.cuda.synchronize()
+        assert_bitexact(dp.owned(out).cpu().numpy(), oracle.run(kind, g, T), f"dist {kind} part_dim={pd}")
 
 @pytest.mark.parametrize("kind,shape,T", [("star2d5", (300, 1030), 19), ("box2d9", (257, 1100), 12),
                                           ("star3d7", (40, 45, 68), 11), ("box3d27", (30, 37, 68), 9)])
