@@ -213,6 +213,15 @@ stencil_status stencil_plan_dist(stencil_plan_t *out, stencil_desc_t global_desc
 stencil_status stencil_dist_local_plan(stencil_plan_t *out, stencil_desc_t global_desc, int64_t T_steps,
                                        const stencil_tile_t *tile, int rank, int nranks, int part_dim);
 
+/* Host-only: the outer rows (hexagonal coordinate z) whose halo lines of ping-pong buffer
+ * `buffer` travel in the exchange before launch k >= 1 of a local plan (stencil_dist_local_plan)
+ * of a slab partitioned along part_dim > 0 with the hexagonal dimension 0 whole: z holds level
+ * L(z) in buffer L(z) % 2 and L(z) - 1 in the other, and the launch reads the older one only where
+ * a z-neighbour is behind.  Writes up to cap rows, *n = their number; *n = -1 if the rule does
+ * not apply (every row travels). */
+stencil_status stencil_dist_halo_rows(stencil_plan_t local_plan, int part_dim, int64_t k, int buffer,
+                                      int32_t *rows, int64_t cap, int64_t *n);
+
 /* The layout of a distributed plan and its launches per run. */
 stencil_status stencil_dist_info(stencil_plan_t plan, stencil_dist_info_t *info);
 

@@ -72,7 +72,7 @@ def _units():
     for src in ["desc.cpp", "plan.cpp", "dist.cpp", "tilemodel.cpp"]:
         units.append((os.path.join(CSRC, src), "cxx", []))
     for src in ["run.cu", "kernels/generic.cu", "kernels/registry.cu", "kernels/fdtd.cu",
-                "kernels/ablation.cu"]:
+                "kernels/ablation.cu", "kernels/halo.cu"]:
         units.append((os.path.join(CSRC, src), "nvcc", []))
     for vid in _variant_ids("fast2d_variants.h", "HEXS_FAST2D_VARIANTS"):
         units.append((os.path.join(KDIR, "fast2d_inst.cu"), "nvcc", [f"-DHEXS_VARIANT={vid}"]))

@@ -29,7 +29,7 @@ SYMBOLS = ["stencil_desc_create", "stencil_desc_deps", "stencil_plan",
            "stencil_plan_launches", "stencil_plan_hexagon", "stencil_plan_schedule_of",
            "stencil_plan_profile", "stencil_plan_profile_read", "stencil_abi_version",
            "stencil_dist_unique_id", "stencil_dist_layout", "stencil_plan_dist", "stencil_dist_info",
-           "stencil_dist_block_plan", "stencil_tile_model", "stencil_dist_local_plan"]
+           "stencil_dist_block_plan", "stencil_tile_model", "stencil_dist_local_plan", "stencil_dist_halo_rows"]
 
 
 class StencilError(RuntimeError):
@@ -119,6 +119,7 @@ def lib() -> ctypes.CDLL:
     L.stencil_dist_block_plan.argtypes = [vp, ctypes.c_int, P(vp)]
     L.stencil_dist_local_plan.argtypes = [P(vp), vp, i64, P(Tile), ctypes.c_int, ctypes.c_int, ctypes.c_int]
     L.stencil_tile_model.argtypes = [vp, ctypes.c_int, ctypes.c_int, ctypes.c_int, ctypes.c_int, P(TileEval)]
+    L.stencil_dist_halo_rows.argtypes = [vp, ctypes.c_int, i64, ctypes.c_int, P(i32), i64, P(i64)]
     for name in SYMBOLS:
         f = getattr(L, name)
         if name not in ("stencil_last_error", "stencil_abi_version"):

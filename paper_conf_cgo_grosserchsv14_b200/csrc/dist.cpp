@@ -42,6 +42,7 @@
 #include <nccl.h>
 
 #include "internal.h"
+#include "kernels/launch.h"
 
 namespace hexs {
 
@@ -120,11 +121,21 @@ struct DistState {
   size_t local_ws = 0;                             // the local plan's workspace (256-B rounded)
   size_t stage_bytes = 0;                          // halo staging area after it (strided partitions)
   char* stage = nullptr;
+  // Needed-state lists (hexagonal dimension 0 whole, a classical dimension partitioned): before
+  // launch k, outer index z (the hexagonal coordinate) holds level L(z) in buffer L(z) % 2 and
+  // L(z)-1 in the other; the next launch reads the older value only where a z-neighbour is
+  // behind (it computes level L(z) from it).  rows[k][b] = the z whose buffer-b halo lines are
+  // read; only those travel (~68 % of both buffers for the (3, 7) hexagon).
+  std::vector<int> row_table;                      // flat: per launch k >= 1, buffer 0 then 1
+  std::vector<std::pair<int64_t, int64_t>> row_span;  // (offset, count) per (k, b)
+  size_t rows_off = 0, rows_bytes = 0;             // the table's copy in the workspace
+  int* rows_dev = nullptr;
   void* comm = nullptr;                            // ncclComm_t
   cudaStream_t comm_stream = nullptr;
   cudaEvent_t ev_ready = nullptr, ev_done = nullptr;
   int comm_dev = -1;
   bool emulate = false;  // HEXS_DIST_EMULATE: a rank's compute alone (no communicator)
+  bool emulate_copies = false;  // HEXS_DIST_EMULATE=2: plus the halo copies, a local copy as the wire
   ~DistState() {
     for (auto& bp : bplans) delete bp.second;
     if (comm) {
@@ -186,6 +197,42 @@ stencil_tile_t dist_local_tile(const Desc& d, const stencil_tile_t* tile, int nr
   return lt;
 }
 
+// The needed-state row lists of a local plan whose hexagonal dimension 0 is whole (a classical
+// dimension part_dim > 0 partitioned): before launch k >= 1, z holds level L(z) in buffer
+// L(z) % 2 and L(z) - 1 in the other; launch k reads the older value only where a z-neighbour is
+// behind (it computes level L(z) from it -- adjacent levels differ by at most one, or the
+// ping-pong WAR order would be broken).  table: per k >= 1, the z of buffer 0, then buffer 1;
+// span[2 (k-1) + b] = (offset, count).  false if the rule does not apply.
+bool halo_rows_table(const Plan& lp, int part_dim, std::vector<int>& table,
+                     std::vector<std::pair<int64_t, int64_t>>& span) {
+  table.clear();
+  span.clear();
+  if (lp.hd != 0 || part_dim <= 0 || lp.executor == EXEC_NAIVE || lp.desc.nfields != 1 || lp.desc.dims < 2)
+    return false;
+  const int64_t Z = lp.desc.ext[0];
+  std::vector<int64_t> lev(Z, 0);  // level each z holds after the launches so far
+  for (size_t k = 0; k < lp.launches.size(); ++k) {
+    const Launch& ln = lp.launches[k];
+    if (k > 0) {
+      for (int b = 0; b < 2; ++b) {
+        const int64_t off = (int64_t)table.size();
+        for (int64_t z = 0; z < Z; ++z) {
+          const bool behind = (z > 0 && lev[z - 1] < lev[z]) || (z + 1 < Z && lev[z + 1] < lev[z]);
+          if ((lev[z] & 1) == b || behind) table.push_back((int)z);
+        }
+        span.push_back({off, (int64_t)table.size() - off});
+      }
+    }
+    for (int a = ln.a_lo; a <= ln.a_hi; ++a)
+      for (int64_t S0 = ln.S0_lo; S0 <= ln.S0_hi; ++S0) {
+        const int64_t i0 = S0 * lp.W - ln.row_off;
+        const int64_t r0 = std::max<int64_t>(i0 + lp.lo[a], 1), r1 = std::min<int64_t>(i0 + lp.hi[a], Z - 2);
+        for (int64_t z = r0; z <= r1; ++z) lev[z] = ln.tau0 + a + 1;
+      }
+  }
+  return true;
+}
+
 // The slab layout of one rank (host only; shared by stencil_dist_layout and stencil_plan_dist).
 stencil_status dist_layout(const Desc& d, int64_t T_steps, const stencil_tile_t* tile, int rank, int nranks,
                            int part_dim, DistLayout* out) {
@@ -230,12 +277,21 @@ stencil_status dist_layout(const Desc& d, int64_t T_steps, const stencil_tile_t*
 
 stencil_status dist_set_workspace(Plan& p, void* dev_ptr, size_t bytes) {
   DistState& s = *p.dist;
-  if (bytes < s.local_ws + s.stage_bytes) return fail(STENCIL_E_OOM, "stencil_plan_set_workspace: workspace too small");
+  if (bytes < s.local_ws + s.stage_bytes + s.rows_bytes)
+    return fail(STENCIL_E_OOM, "stencil_plan_set_workspace: workspace too small");
   for (auto& bp : s.bplans) {
     bp.second->ws = dev_ptr;
     bp.second->ws_size = s.local_ws;
   }
   s.stage = s.stage_bytes ? static_cast<char*>(dev_ptr) + s.local_ws : nullptr;
+  s.rows_dev = nullptr;
+  if (!s.row_table.empty()) {  // the needed-state lists, uploaded once per workspace
+    s.rows_dev = reinterpret_cast<int*>(static_cast<char*>(dev_ptr) + s.rows_off);
+    const cudaError_t e = cudaMemcpy(s.rows_dev, s.row_table.data(), s.row_table.size() * sizeof(int),
+                                     cudaMemcpyHostToDevice);
+    if (e != cudaSuccess)
+      return fail(STENCIL_E_CUDA, std::string("stencil_plan_set_workspace: halo row lists: ") + cudaGetErrorString(e));
+  }
   return STENCIL_OK;
 }
 
@@ -244,13 +300,18 @@ stencil_status dist_set_workspace(Plan& p, void* dev_ptr, size_t bytes) {
 // partition of dimension 0 sends contiguous planes; a deeper one is strided (n_outer blocks of
 // G lines, local_n lines apart) and goes through the staging area: packed by 2-D copies, sent,
 // received, unpacked -- all on the communication stream.
-static stencil_status exchange(DistState& s, void* const* bufs, cudaStream_t stream) {
-  NcclApi* a = nccl_api();
-  if (!a) return fail(STENCIL_E_NCCL, "NCCL unavailable");
+static stencil_status exchange(DistState& s, int64_t k, void* const* bufs, cudaStream_t stream) {
+  NcclApi* a = s.emulate_copies ? nullptr : nccl_api();
+  if (!a && !s.emulate_copies) return fail(STENCIL_E_NCCL, "NCCL unavailable");
   const DistLayout& L = s.lay;
   const int64_t G = L.ghost, local_n = L.loc_hi - L.loc_lo;
   const size_t chunk = (size_t)G * s.line_bytes;  // one outer block of a halo
-  const size_t n = chunk * (size_t)s.n_outer;     // one halo
+  const size_t n = chunk * (size_t)s.n_outer;     // one halo (staging slot size)
+  // rows of buffer b this exchange moves (all, or the needed-state list of launch k)
+  const bool listed = s.rows_dev != nullptr && k >= 1 && (size_t)(2 * (k - 1) + 1) < s.row_span.size();
+  auto nrows = [&](int b) { return listed ? (size_t)s.row_span[2 * (k - 1) + b].second : (size_t)s.n_outer; };
+  auto rows = [&](int b) -> const int* { return listed ? s.rows_dev + s.row_span[2 * (k - 1) + b].first : nullptr; };
+  auto msg = [&](int b) { return chunk * nrows(b); };
   const size_t pitch = (size_t)local_n * s.line_bytes;
   const bool strided = s.n_outer > 1;
   if (strided && !s.stage) return fail(STENCIL_E_INVALID, "stencil_run: workspace not set (halo staging)");
@@ -264,40 +325,56 @@ static stencil_status exchange(DistState& s, void* const* bufs, cudaStream_t str
   // staging layout per buffer b: [send lo][send hi][recv lo][recv hi]
   auto stg = [&](int b, int slot) { return s.stage + ((size_t)b * 4 + slot) * n; };
   auto at = [&](int b, int64_t idx) { return static_cast<char*>(bufs[b]) + (size_t)idx * s.line_bytes; };
+  // strided halos: one gather launch for every region of this exchange (kernels/halo.cu)
   if (strided) {
-    for (int b = 0; b < 2 && e == cudaSuccess; ++b) {
-      if (lo_nb) e = cudaMemcpy2DAsync(stg(b, 0), chunk, at(b, own0), pitch, chunk, s.n_outer, cudaMemcpyDeviceToDevice, cs);
-      if (hi_nb && e == cudaSuccess)
-        e = cudaMemcpy2DAsync(stg(b, 1), chunk, at(b, own1 - G), pitch, chunk, s.n_outer, cudaMemcpyDeviceToDevice, cs);
+    HaloCopyArgs pk{};
+    for (int b = 0; b < 2; ++b) {
+      if (nrows(b) == 0) continue;
+      if (lo_nb) pk.reg[pk.n++] = HaloRegion{stg(b, 0), at(b, own0), chunk, pitch, chunk, nrows(b), rows(b), nullptr};
+      if (hi_nb) pk.reg[pk.n++] = HaloRegion{stg(b, 1), at(b, own1 - G), chunk, pitch, chunk, nrows(b), rows(b), nullptr};
     }
+    e = launch_halo_copy(pk, cs);
     if (e != cudaSuccess) return fail(STENCIL_E_CUDA, std::string("stencil_run: halo pack: ") + cudaGetErrorString(e));
   }
-  ncclResult_t r = a->GroupStart();
-  if (r != ncclSuccess) return nccl_fail(a, r, "ncclGroupStart");
-  for (int b = 0; b < 2; ++b) {
-    if (lo_nb) {
-      a->Send(strided ? stg(b, 0) : at(b, own0), n, ncclChar, L.rank - 1, comm, cs);
-      a->Recv(strided ? stg(b, 2) : at(b, own0 - G), n, ncclChar, L.rank - 1, comm, cs);
-    }
-    if (hi_nb) {
-      a->Send(strided ? stg(b, 1) : at(b, own1 - G), n, ncclChar, L.rank + 1, comm, cs);
-      a->Recv(strided ? stg(b, 3) : at(b, own1), n, ncclChar, L.rank + 1, comm, cs);
+  if (s.emulate_copies) {  // single-GPU projection: the wire is a device-local copy
+    for (int b = 0; b < 2 && e == cudaSuccess; ++b) {
+      if (lo_nb && msg(b))
+        e = cudaMemcpyAsync(strided ? stg(b, 2) : at(b, own0 - G), strided ? stg(b, 0) : at(b, own0), msg(b),
+                            cudaMemcpyDeviceToDevice, cs);
+      if (hi_nb && msg(b) && e == cudaSuccess)
+        e = cudaMemcpyAsync(strided ? stg(b, 3) : at(b, own1), strided ? stg(b, 1) : at(b, own1 - G), msg(b),
+                            cudaMemcpyDeviceToDevice, cs);
     }
   }
-  r = a->GroupEnd();
+  ncclResult_t r = s.emulate_copies ? ncclSuccess : a->GroupStart();
+  if (r != ncclSuccess) return nccl_fail(a, r, "ncclGroupStart");
+  for (int b = 0; b < 2 && !s.emulate_copies; ++b) {
+    if (msg(b) == 0) continue;
+    if (lo_nb) {
+      a->Send(strided ? stg(b, 0) : at(b, own0), msg(b), ncclChar, L.rank - 1, comm, cs);
+      a->Recv(strided ? stg(b, 2) : at(b, own0 - G), msg(b), ncclChar, L.rank - 1, comm, cs);
+    }
+    if (hi_nb) {
+      a->Send(strided ? stg(b, 1) : at(b, own1 - G), msg(b), ncclChar, L.rank + 1, comm, cs);
+      a->Recv(strided ? stg(b, 3) : at(b, own1), msg(b), ncclChar, L.rank + 1, comm, cs);
+    }
+  }
+  r = s.emulate_copies ? ncclSuccess : a->GroupEnd();
   if (r != ncclSuccess) return nccl_fail(a, r, "ncclGroupEnd");
   if (strided) {
-    for (int b = 0; b < 2 && e == cudaSuccess; ++b) {
-      if (lo_nb) e = cudaMemcpy2DAsync(at(b, own0 - G), pitch, stg(b, 2), chunk, chunk, s.n_outer, cudaMemcpyDeviceToDevice, cs);
-      if (hi_nb && e == cudaSuccess)
-        e = cudaMemcpy2DAsync(at(b, own1), pitch, stg(b, 3), chunk, chunk, s.n_outer, cudaMemcpyDeviceToDevice, cs);
+    HaloCopyArgs uk{};
+    for (int b = 0; b < 2; ++b) {
+      if (nrows(b) == 0) continue;
+      if (lo_nb) uk.reg[uk.n++] = HaloRegion{at(b, own0 - G), stg(b, 2), pitch, chunk, chunk, nrows(b), nullptr, rows(b)};
+      if (hi_nb) uk.reg[uk.n++] = HaloRegion{at(b, own1), stg(b, 3), pitch, chunk, chunk, nrows(b), nullptr, rows(b)};
     }
+    e = launch_halo_copy(uk, cs);
     if (e != cudaSuccess) return fail(STENCIL_E_CUDA, std::string("stencil_run: halo unpack: ") + cudaGetErrorString(e));
   }
   e = cudaEventRecord(s.ev_done, cs);
   if (e == cudaSuccess) e = cudaStreamWaitEvent(stream, s.ev_done, 0);
   if (e != cudaSuccess) return fail(STENCIL_E_CUDA, std::string("stencil_run: halo ordering: ") + cudaGetErrorString(e));
-  if (a->CommGetAsyncError) {
+  if (a && a->CommGetAsyncError && comm) {
     ncclResult_t ae = ncclSuccess;
     if (a->CommGetAsyncError(comm, &ae) == ncclSuccess && ae != ncclSuccess && ae != ncclInProgress)
       return nccl_fail(a, ae, "NCCL async error");
@@ -306,10 +383,10 @@ static stencil_status exchange(DistState& s, void* const* bufs, cudaStream_t str
 }
 
 // pre_launch hook of the local plan: refresh both buffers' ghost planes
-static stencil_status ghost_hook(void* ctx, int64_t /*k*/, void* const* bufs, void* stream) {
+static stencil_status ghost_hook(void* ctx, int64_t k, void* const* bufs, void* stream) {
   DistState& s = *static_cast<DistState*>(ctx);
-  if (s.lay.nranks <= 1 || s.emulate) return STENCIL_OK;
-  return exchange(s, bufs, static_cast<cudaStream_t>(stream));
+  if (s.lay.nranks <= 1 || (s.emulate && !s.emulate_copies)) return STENCIL_OK;
+  return exchange(s, k, bufs, static_cast<cudaStream_t>(stream));
 }
 
 stencil_status run_dist(Plan& p, const void* const* in, void* const* out, void* stream_) {
@@ -433,6 +510,7 @@ stencil_status stencil_plan_dist(stencil_plan_t* out, stencil_desc_t global_desc
   // communicator, no exchanges (the ghost planes keep their initial values, so results are not
   // the global ones); it measures a rank's compute for scaling projections on a single GPU
   s->emulate = std::getenv("HEXS_DIST_EMULATE") && std::atoi(std::getenv("HEXS_DIST_EMULATE")) != 0;
+  s->emulate_copies = s->emulate && std::atoi(std::getenv("HEXS_DIST_EMULATE")) == 2;
   if (!s->emulate) {  // (also for one rank: the same NCCL bootstrap path, no exchange ever runs)
     NcclApi* a = nccl_api();
     if (!a) return fail(STENCIL_E_NCCL, "stencil_plan_dist: NCCL unavailable");
@@ -463,7 +541,14 @@ stencil_status stencil_plan_dist(stencil_plan_t* out, stencil_desc_t global_desc
   s->local_ws = (ws + 255) / 256 * 256;
   // strided partitions: staging for both buffers' 2 send + 2 receive halos
   s->stage_bytes = s->n_outer > 1 && nranks > 1 ? 8 * (size_t)L.ghost * s->line_bytes * (size_t)s->n_outer : 0;
-  p->ws_bytes = s->local_ws + s->stage_bytes;
+  // needed-state row lists: the hexagonal dimension 0 whole (its coordinate is the outer index
+  // of the halo blocks), a classical dimension partitioned
+  Plan* lp0 = s->bplans.empty() ? nullptr : s->bplans[0].second;
+  if (s->stage_bytes && lp0 && halo_rows_table(*lp0, pd, s->row_table, s->row_span)) {
+    s->rows_off = s->local_ws + s->stage_bytes;
+    s->rows_bytes = (s->row_table.size() * sizeof(int) + 255) / 256 * 256;
+  }
+  p->ws_bytes = s->local_ws + s->stage_bytes + s->rows_bytes;
   p->dist = s.release();
   *out = reinterpret_cast<stencil_plan_t>(p);
   return STENCIL_OK;
@@ -492,6 +577,26 @@ stencil_status stencil_dist_local_plan(stencil_plan_t* out, stencil_desc_t globa
   st = build_plan(local, T_steps, &lt, &p, origin);
   if (st != STENCIL_OK) return st;
   *out = reinterpret_cast<stencil_plan_t>(p);
+  return STENCIL_OK;
+}
+
+stencil_status stencil_dist_halo_rows(stencil_plan_t local_plan, int part_dim, int64_t k, int buffer, int32_t* rows,
+                                     int64_t cap, int64_t* n) {
+  clear_error();
+  Plan* p = as_plan(local_plan);
+  if (!p || p->dist || !n || buffer < 0 || buffer > 1 || k < 1)
+    return fail(STENCIL_E_INVALID, "stencil_dist_halo_rows: bad arguments");
+  std::vector<int> table;
+  std::vector<std::pair<int64_t, int64_t>> span;
+  if (!halo_rows_table(*p, part_dim, table, span)) {
+    *n = -1;  // the rule does not apply: every outer row travels
+    return STENCIL_OK;
+  }
+  if ((size_t)(2 * (k - 1) + buffer) >= span.size()) return fail(STENCIL_E_INVALID, "stencil_dist_halo_rows: k out of range");
+  const auto sp = span[2 * (k - 1) + buffer];
+  *n = sp.second;
+  if (rows)
+    for (int64_t i = 0; i < sp.second && i < cap; ++i) rows[i] = table[sp.first + i];
   return STENCIL_OK;
 }
 

@@ -147,4 +147,20 @@ struct AblArgs {
 cudaError_t launch_ablation(int cfg, int kind, const AblArgs& a, cudaStream_t s);
 size_t ablation_smem_bytes(int cfg, int W, int YB, int XP);
 
+// Slab-mode halo staging (kernels/halo.cu): up to kMaxHaloRegions strided 2-D copies in one
+// launch (rows x width bytes, widths / pitches / pointers 16-B aligned).
+constexpr int kMaxHaloRegions = 8;
+struct HaloRegion {
+  char* dst;
+  const char* src;
+  size_t dpitch, spitch, width, rows;
+  const int* src_rows;  // optional row index lists (gather / scatter); nullptr = row i
+  const int* dst_rows;
+};
+struct HaloCopyArgs {
+  int n;
+  HaloRegion reg[kMaxHaloRegions];
+};
+cudaError_t launch_halo_copy(const HaloCopyArgs& a, cudaStream_t s);
+
 }  // namespace hexs

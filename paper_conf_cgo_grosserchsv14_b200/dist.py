@@ -114,28 +114,47 @@ def local_plan(kind: str, global_ext: Sequence[int], T: int, rank: int, nranks: 
     return Plan._adopt(Stencil(kind, lay.local_ext, dtype=dtype), h, T), lay
 
 
-def exchange_halos(local: torch.Tensor, lay: Layout, group=None) -> None:
+def halo_rows(plan, part_dim: int, k: int, buffer: int) -> Optional[List[int]]:
+    """The outer rows whose halo lines of `buffer` travel before launch k of a local plan
+    (stencil_dist_halo_rows), or None when every row travels."""
+    n = ctypes.c_int64()
+    check(lib().stencil_dist_halo_rows(plan._h, int(part_dim), int(k), int(buffer), None, 0, ctypes.byref(n)))
+    if n.value < 0:
+        return None
+    arr = (ctypes.c_int32 * max(1, n.value))()
+    check(lib().stencil_dist_halo_rows(plan._h, int(part_dim), int(k), int(buffer), arr, n.value, ctypes.byref(n)))
+    return list(arr[:n.value])
+
+
+def exchange_halos(local: torch.Tensor, lay: Layout, group=None, rows: Optional[Sequence[int]] = None) -> None:
     """The library's halo step over torch.distributed (for CPU/gloo tests of the protocol):
     send my first / last G owned indices of the partitioned dimension down / up, receive the
-    neighbours' into my ghosts (strided slabs through contiguous staging, as the library does)."""
+    neighbours' into my ghosts (strided slabs through contiguous staging, as the library does);
+    `rows`: only these outer (dimension-0) rows travel (the library's needed-state lists)."""
     G = lay.ghost
     lo, hi = lay.own_local
+    sel = (lambda t: t) if rows is None else (lambda t: t[list(rows)])
     ops, unpack = [], []
     if lay.rank > 0:
-        rl = torch.empty_like(lay.take(local, lo - G, lo).contiguous())
-        ops.append(dist.P2POp(dist.isend, lay.take(local, lo, lo + G).contiguous(), lay.rank - 1, group))
+        rl = torch.empty_like(sel(lay.take(local, lo - G, lo)).contiguous())
+        ops.append(dist.P2POp(dist.isend, sel(lay.take(local, lo, lo + G)).contiguous(), lay.rank - 1, group))
         ops.append(dist.P2POp(dist.irecv, rl, lay.rank - 1, group))
         unpack.append((lo - G, lo, rl))
     if lay.rank < lay.nranks - 1:
-        rh = torch.empty_like(lay.take(local, hi, hi + G).contiguous())
-        ops.append(dist.P2POp(dist.isend, lay.take(local, hi - G, hi).contiguous(), lay.rank + 1, group))
+        rh = torch.empty_like(sel(lay.take(local, hi, hi + G)).contiguous())
+        ops.append(dist.P2POp(dist.isend, sel(lay.take(local, hi - G, hi)).contiguous(), lay.rank + 1, group))
         ops.append(dist.P2POp(dist.irecv, rh, lay.rank + 1, group))
         unpack.append((hi, hi + G, rh))
     if ops:
         for req in dist.batch_isend_irecv(ops):
             req.wait()
     for a, b, buf in unpack:
-        lay.take(local, a, b).copy_(buf)
+        if rows is None:
+            lay.take(local, a, b).copy_(buf)
+        else:
+            view = lay.take(local, a, b)
+            for i, z in enumerate(rows):
+                view[z].copy_(buf[i])
 
 
 def run_protocol(bufs: Sequence[torch.Tensor], lay: Layout, plan, execute_launch: Callable, group=None) -> None:
@@ -144,8 +163,8 @@ def run_protocol(bufs: Sequence[torch.Tensor], lay: Layout, plan, execute_launch
     planes of both ping-pong buffers (but before the first), then run the launch."""
     for k, ln in enumerate(plan.launches()):
         if k > 0 and lay.nranks > 1:
-            for b in bufs:
-                exchange_halos(b, lay, group)
+            for bi, b in enumerate(bufs):
+                exchange_halos(b, lay, group, halo_rows(plan, lay.part_dim, k, bi))
         execute_launch(ln, bufs)
 
 
@@ -164,7 +183,7 @@ class DistPlan:
         emu = os.environ.get("HEXS_DIST_EMULATE_RANK")  # "r/P": play rank r of P alone (projection)
         if emu:
             r, P = (int(x) for x in emu.split("/"))
-            os.environ["HEXS_DIST_EMULATE"] = "1"
+            os.environ.setdefault("HEXS_DIST_EMULATE", "1")  # "2": with the halo copies
             self.rank, self.nranks = r, P
         self._d = _desc(kind, self.global_ext, dtype)
         uid = (ctypes.c_char * 128)()

@@ -146,3 +146,37 @@ def test_layout_properties():
         hdist.layout("star2d5", (10, 10), 40, 0, 4)
     with pytest.raises(StencilError):
         hdist.layout("fdtd2d", (40, 40), 10, 0, 2)
+
+
+def test_halo_rows_needed_state():
+    """stencil_dist_halo_rows: before every launch each z travels in the buffer of its current
+    level, and in the other one exactly where a z-neighbour is one level behind; for the (3, 7)
+    hexagon that is ~68 % of both buffers' halo lines (the 1024^3 slabs' exchange volume)."""
+    ext, T = (1024, 1024, 1024), 256
+    plan, lay = hdist.local_plan("star3d7", ext, T, 3, 8)
+    assert lay.part_dim == 1 and (plan.info["h"], plan.info["w0"]) == (3, 7)
+    lo, hi = plan.hexagon()
+    W = plan.info["W"]
+    lev = np.zeros(ext[0], dtype=np.int64)
+    total = moved = 0
+    for k, ln in enumerate(plan.launches()):
+        if k > 0:
+            rows = [hdist.halo_rows(plan, 1, k, b) for b in (0, 1)]
+            for b in (0, 1):
+                exp = [z for z in range(ext[0])
+                       if lev[z] % 2 == b or (z > 0 and lev[z - 1] < lev[z]) or (z + 1 < ext[0] and lev[z + 1] < lev[z])]
+                assert rows[b] == exp
+            assert set(rows[0]) | set(rows[1]) == set(range(ext[0]))
+            total += 2 * ext[0]
+            moved += len(rows[0]) + len(rows[1])
+        for a in range(ln["a_lo"], ln["a_hi"] + 1):
+            for S0 in range(ln["S0_lo"], ln["S0_hi"] + 1):
+                i0 = S0 * W - ln["row_off"]
+                r0, r1 = max(i0 + lo[a], 1), min(i0 + hi[a], ext[0] - 2)
+                if r0 <= r1:
+                    lev[r0:r1 + 1] = ln["tau0"] + a + 1
+            assert np.all(np.abs(np.diff(lev[1:-1])) <= 1)  # adjacent levels differ by <= 1 (ping-pong WAR)
+    assert 0.6 < moved / total < 0.75
+    # the hexagonal dimension partitioned: every plane travels
+    p0, _ = hdist.local_plan("star3d7", (64, 48, 40), 20, 1, 2, part_dim=0)
+    assert hdist.halo_rows(p0, 0, 1, 0) is None
