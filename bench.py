@@ -157,15 +157,16 @@ KERNEL_NAMES = {"fast2d": "fast2d_kernel (2D register wavefront)", "fdtd": "fdtd
 
 def measured_traffic(cfg, tile):
     """DRAM bytes per launch of the phase kernel from the committed ncu launch list
-    (profiles/round1/traffic_<cfg>.json: dram__bytes_read.sum + dram__bytes_write.sum summed
-    over every launch of one stencil_run, divided by the launch count), or None."""
-    p = os.path.join(ROOT, "profiles", "round1", f"traffic_{cfg}.json")
-    if not os.path.exists(p):
-        return None
-    d = json.load(open(p))
-    if d.get("tile") != tile:
-        return None
-    return d["dram_bytes_per_launch"]
+    (profiles/round2/traffic_<cfg>.json, else round1's: dram__bytes_read.sum +
+    dram__bytes_write.sum summed over every launch of one stencil_run, divided by the launch
+    count), or None."""
+    for rnd in ("round2", "round1"):
+        p = os.path.join(ROOT, "profiles", rnd, f"traffic_{cfg}.json")
+        if os.path.exists(p):
+            d = json.load(open(p))
+            if d.get("tile") == tile:
+                return d["dram_bytes_per_launch"], f"profiles/{rnd}/traffic_{cfg}.json", d.get("l2_bytes_per_update")
+    return None, None, None
 
 
 def cpu_baseline(kind, ext, target_s=12.0):
@@ -421,6 +422,7 @@ def run_gpu(args, cfg):
     naive_gups = updates / (n0.elapsed_time(n1) * 1e-3) / 1e9
     cpu = None if args.no_cpu else cpu_baseline(kind, ext)
     tiled_roof = peak * 1e9 / bpu / 1e9  # GUp/s if HBM-bound at the tiled bytes/update
+    traffic = measured_traffic(cfg, {"h": info["h"], "w0": info["w0"]})
     line = {
         "metric": METRIC, "value": value, "unit": "GStencil-updates/s", "n_gpus": 1,
         "steps": args.steps, "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True,
@@ -430,9 +432,10 @@ def run_gpu(args, cfg):
                    "l2": l2_note},
         "roofline": {"bound": "hbm", "achieved": achieved_gbs, "peak": peak, "unit": "GB/s",
                      "frac": achieved_gbs / peak,
-                     "traffic": measured_traffic(cfg, {"h": info["h"], "w0": info["w0"]}),
+                     "traffic": traffic[0],
                      "traffic_source": "ncu dram__bytes_read.sum+dram__bytes_write.sum per launch "
-                                       f"(profiles/round1/traffic_{cfg}.json)",
+                                       f"({traffic[1]})",
+                     "l2_bytes_per_update": traffic[2],
                      "alg_bytes_per_launch": alg_bytes_per_launch, "peak_source": peak_src,
                      "kernel": KERNEL_NAMES[plan.executor_name],
                      "bytes_per_update": bpu, "avg_launch_ms": avg_launch_ms,

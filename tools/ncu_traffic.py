@@ -5,7 +5,9 @@ On the GPU box (one stencil_run, every launch of the phase kernel, cold-cache, s
       --clock-control none -k regex:KERNEL --csv --log-file gpurun_out/launches_CFG.csv \
       python tools/run_once.py CFG 1
 Here: python tools/ncu_traffic.py CFG gpurun_out/launches_CFG.csv
-  -> profiles/round1/traffic_CFG.json (read by bench.py for roofline.traffic)."""
+  -> profiles/round2/traffic_CFG.json (read by bench.py for roofline.traffic).
+Also records L2 bytes per update (lts__t_bytes.sum) and the CTAs-per-launch histogram
+(launch__grid_size) when the launch list carries them."""
 import csv
 import json
 import os
@@ -30,20 +32,29 @@ def main(cfg, path):
         d = per.setdefault(r[idi], {"kernel": r[ki]})
         d[r[mi]] = float(r[vi].replace(",", "")) * scale.get(r[ui], 1.0)
     launches = list(per.values())
-    kind, ext, T, _ = bench.CONFIGS[cfg]
+    kind, ext, T, _ = bench.CONFIGS[cfg][:4]
     plan = Plan(Stencil(kind, ext), T)
     info = plan.info
     tot_b = sum(l["dram__bytes_read.sum"] + l["dram__bytes_write.sum"] for l in launches)
     tot_t = sum(l["gpu__time_duration.sum"] for l in launches)
     bpu = bench.bytes_per_update_tiled(info, 4, plan)
+    hist = {}
+    for l in launches:
+        if "launch__grid_size" in l:
+            g = int(l["launch__grid_size"])
+            hist[g] = hist.get(g, 0) + 1
+    lts = sum(l.get("lts__t_bytes.sum", 0.0) for l in launches)
     out = {"config": cfg, "kernel": launches[0]["kernel"][:120], "launches": len(launches),
            "plan_launches": info["n_launches"], "tile": {"h": info["h"], "w0": info["w0"]},
            "dram_bytes_total": tot_b, "dram_bytes_per_launch": tot_b / len(launches),
            "dram_bytes_per_update": tot_b / info["updates"],
            "algorithmic_bytes_per_update": bpu,
            "kernel_time_total_s_cold_serialised": tot_t,
+           "l2_bytes_per_update": lts / info["updates"] if lts else None,
+           "ctas_per_launch_histogram": {str(k): v for k, v in sorted(hist.items())},
            "source": os.path.basename(path)}
-    dst = os.path.join(ROOT, "profiles", "round1", f"traffic_{cfg}.json")
+    os.makedirs(os.path.join(ROOT, "profiles", "round2"), exist_ok=True)
+    dst = os.path.join(ROOT, "profiles", "round2", f"traffic_{cfg}.json")
     json.dump(out, open(dst, "w"), indent=1)
     print(json.dumps(out, indent=1))
 

@@ -14,7 +14,7 @@ tile = {}
 if len(sys.argv) > 4:
     tile = {"h": int(sys.argv[3]), "w0": int(sys.argv[4])}
 execu = os.environ.get("HEXS_EXEC", "auto")
-kind, ext, T, _ = bench.CONFIGS[cfg]
+kind, ext, T, _ = bench.CONFIGS[cfg][:4]
 fields = bench.make_inputs(kind, ext)
 plan = Plan(Stencil(kind, ext), T, executor=execu, **tile)
 xs = [torch.from_numpy(f).cuda() for f in fields]
