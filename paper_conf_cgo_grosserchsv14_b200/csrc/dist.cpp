@@ -251,12 +251,8 @@ stencil_status dist_layout(const Desc& d, int64_t T_steps, const stencil_tile_t*
   const int64_t base = N0 / nranks, extra = N0 % nranks;
   L.own_lo = rank * base + std::min<int64_t>(rank, extra);
   L.own_hi = L.own_lo + base + (rank < extra ? 1 : 0);
-  // time block: a multiple of the hexagon height 2h+2 of the local plans' tile (one time tile
-  // by default, more while the ghost planes stay within ~10% of the owned ones);
-  // HEXS_TIME_BLOCK overrides
   const stencil_tile_t lt = dist_local_tile(d, tile, nranks);
   const int h = lt.h;
-  const int64_t H = 2 * (int64_t)h + 2;
   const int64_t owned = L.own_hi - L.own_lo;
   // one exchange per phase launch: a launch spans at most 2h+2 levels (one time tile)
   const int64_t D = 2 * (int64_t)h + 2;
