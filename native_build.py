@@ -72,8 +72,10 @@ def _units():
     for src in ["desc.cpp", "plan.cpp", "dist.cpp", "tilemodel.cpp"]:
         units.append((os.path.join(CSRC, src), "cxx", []))
     for src in ["run.cu", "kernels/generic.cu", "kernels/registry.cu", "kernels/fdtd.cu",
-                "kernels/ablation.cu", "kernels/halo.cu"]:
+                "kernels/ablation.cu"]:
         units.append((os.path.join(CSRC, src), "nvcc", []))
+    # the halo kernels use NCCL's device API (symmetric-window LSA pointers): nccl_device.h
+    units.append((os.path.join(CSRC, "kernels/halo.cu"), "nvcc", ["-I" + _nccl_include()]))
     for vid in _variant_ids("fast2d_variants.h", "HEXS_FAST2D_VARIANTS"):
         units.append((os.path.join(KDIR, "fast2d_inst.cu"), "nvcc", [f"-DHEXS_VARIANT={vid}"]))
     for vid in _variant_ids("fast3d_variants.h", "HEXS_FAST3D_VARIANTS"):
@@ -83,7 +85,8 @@ def _units():
     out = []
     for src, tool, extra in units:
         key = _deps_hash([src] + headers) + hashlib.sha1(" ".join(extra).encode()).hexdigest()[:8]
-        name = os.path.relpath(src, CSRC).replace("/", "_") + ("_" + "_".join(e.split("=")[-1] for e in extra) if extra else "")
+        tags = [e.split("=")[-1] for e in extra if "=" in e]
+        name = os.path.relpath(src, CSRC).replace("/", "_") + ("_" + "_".join(tags) if tags else "")
         out.append((src, tool, extra, os.path.join(OBJ, f"{name}.{key}.o")))
     return out
 

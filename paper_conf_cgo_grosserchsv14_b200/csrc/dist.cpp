@@ -33,7 +33,9 @@
 #include <algorithm>
 #include <cstdlib>
 #include <cstring>
+#include <map>
 #include <memory>
+#include <mutex>
 #include <new>
 #include <string>
 #include <vector>
@@ -59,6 +61,11 @@ struct NcclApi {
   ncclResult_t (*Recv)(void*, size_t, ncclDataType_t, int, ncclComm_t, cudaStream_t) = nullptr;
   const char* (*GetErrorString)(ncclResult_t) = nullptr;
   ncclResult_t (*CommGetAsyncError)(ncclComm_t, ncclResult_t*) = nullptr;
+  // symmetric memory (NCCL >= 2.27): device-initiated halo stores through LSA pointers
+  ncclResult_t (*MemAlloc)(void**, size_t) = nullptr;
+  ncclResult_t (*MemFree)(void*) = nullptr;
+  ncclResult_t (*WindowRegister)(ncclComm_t, void*, size_t, ncclWindow_t*, int) = nullptr;
+  ncclResult_t (*WindowDeregister)(ncclComm_t, ncclWindow_t) = nullptr;
   std::string error;
 };
 
@@ -90,6 +97,10 @@ NcclApi* nccl_api() {
   api.Recv = reinterpret_cast<decltype(api.Recv)>(sym("ncclRecv"));
   api.GetErrorString = reinterpret_cast<decltype(api.GetErrorString)>(sym("ncclGetErrorString"));
   api.CommGetAsyncError = reinterpret_cast<decltype(api.CommGetAsyncError)>(sym("ncclCommGetAsyncError"));
+  api.MemAlloc = reinterpret_cast<decltype(api.MemAlloc)>(sym("ncclMemAlloc"));
+  api.MemFree = reinterpret_cast<decltype(api.MemFree)>(sym("ncclMemFree"));
+  api.WindowRegister = reinterpret_cast<decltype(api.WindowRegister)>(sym("ncclCommWindowRegister"));
+  api.WindowDeregister = reinterpret_cast<decltype(api.WindowDeregister)>(sym("ncclCommWindowDeregister"));
   if (!api.GetUniqueId || !api.CommInitRank || !api.CommDestroy || !api.GroupStart || !api.GroupEnd ||
       !api.Send || !api.Recv || !api.GetErrorString) {
     api.error = "libnccl.so.2 lacks a required symbol";
@@ -130,13 +141,27 @@ struct DistState {
   std::vector<std::pair<int64_t, int64_t>> row_span;  // (offset, count) per (k, b)
   size_t rows_off = 0, rows_bytes = 0;             // the table's copy in the workspace
   int* rows_dev = nullptr;
+  // Device-initiated exchange (default for nranks > 1 when NCCL symmetric windows work, or in
+  // loopback mode HEXS_DIST_LOOPBACK=1: the ranks are plans of one process on one device): each
+  // rank owns a receive area [slot k%2][side: from lower, from upper][buffer] x halo bytes + two
+  // flags + a block counter; the sender's kernel stores straight into the neighbour's area.
+  bool p2p = false, loopback = false;
+  char* recv = nullptr;
+  size_t recv_bytes = 0, recv_halo = 0, flag_off = 0;
+  void* win = nullptr;                      // ncclWindow_t of `recv`
+  char* peer_recv[2] = {nullptr, nullptr};  // the lower / upper neighbour's receive area
+  unsigned int done_count = 0;              // host mirror of the send kernel's block counter
+  int64_t runs = 0;                         // completed stencil_runs (flag sequence base)
+  std::string group;                        // loopback registry key
   void* comm = nullptr;                            // ncclComm_t
   cudaStream_t comm_stream = nullptr;
   cudaEvent_t ev_ready = nullptr, ev_done = nullptr;
   int comm_dev = -1;
   bool emulate = false;  // HEXS_DIST_EMULATE: a rank's compute alone (no communicator)
   bool emulate_copies = false;  // HEXS_DIST_EMULATE=2: plus the halo copies, a local copy as the wire
-  ~DistState() {
+  ~DistState();
+  void release_p2p();
+  void destroy_rest() {
     for (auto& bp : bplans) delete bp.second;
     if (comm) {
       if (NcclApi* a = nccl_api()) a->CommDestroy(static_cast<ncclComm_t>(comm));
@@ -151,6 +176,34 @@ struct DistState {
     return nullptr;
   }
 };
+
+// loopback registry: the ranks of one group (keyed by the unique id) in this process
+static std::mutex g_loop_mu;
+static std::map<std::string, std::vector<DistState*>> g_loop;
+
+void DistState::release_p2p() {
+  if (loopback && !group.empty()) {
+    std::lock_guard<std::mutex> lk(g_loop_mu);
+    auto it = g_loop.find(group);
+    if (it != g_loop.end()) {
+      for (auto& q : it->second)
+        if (q == this) q = nullptr;
+    }
+  }
+  if (recv) {
+    NcclApi* a = nccl_api();
+    if (win && a && a->WindowDeregister) a->WindowDeregister(static_cast<ncclComm_t>(comm), static_cast<ncclWindow_t>(win));
+    if (loopback) cudaFree(recv);
+    else if (a && a->MemFree) a->MemFree(recv);
+  }
+  recv = nullptr;
+  win = nullptr;
+}
+
+DistState::~DistState() {
+  release_p2p();
+  destroy_rest();
+}
 
 void dist_free(DistState* d) { delete d; }
 
@@ -280,9 +333,11 @@ stencil_status dist_set_workspace(Plan& p, void* dev_ptr, size_t bytes) {
     bp.second->ws_size = s.local_ws;
   }
   s.stage = s.stage_bytes ? static_cast<char*>(dev_ptr) + s.local_ws : nullptr;
+  int* const rows_at = s.row_table.empty() ? nullptr : reinterpret_cast<int*>(static_cast<char*>(dev_ptr) + s.rows_off);
+  if (rows_at && rows_at == s.rows_dev) return STENCIL_OK;  // same workspace: the lists are there
   s.rows_dev = nullptr;
-  if (!s.row_table.empty()) {  // the needed-state lists, uploaded once per workspace
-    s.rows_dev = reinterpret_cast<int*>(static_cast<char*>(dev_ptr) + s.rows_off);
+  if (rows_at) {  // the needed-state lists, uploaded once per workspace (a synchronous copy)
+    s.rows_dev = rows_at;
     const cudaError_t e = cudaMemcpy(s.rows_dev, s.row_table.data(), s.row_table.size() * sizeof(int),
                                      cudaMemcpyHostToDevice);
     if (e != cudaSuccess)
@@ -379,9 +434,73 @@ static stencil_status exchange(DistState& s, int64_t k, void* const* bufs, cudaS
 }
 
 // pre_launch hook of the local plan: refresh both buffers' ghost planes
+// The device-initiated exchange before launch k: my halo lines go straight into the neighbours'
+// receive areas (slot k % 2) by a kernel whose last block publishes the sequence number into
+// their flags; a second kernel waits for my neighbours' sequence numbers and scatters my receive
+// area into my ghost lines.  Both on the compute stream (no host synchronisation, no NCCL call).
+static stencil_status exchange_p2p(DistState& s, int64_t k, void* const* bufs, cudaStream_t stream) {
+  const DistLayout& L = s.lay;
+  if (s.loopback && (!s.peer_recv[0] && L.rank > 0 || !s.peer_recv[1] && L.rank < L.nranks - 1)) {
+    std::lock_guard<std::mutex> lk(g_loop_mu);  // resolve the neighbours of this process
+    auto& v = g_loop[s.group];
+    if (L.rank > 0 && (int)v.size() > L.rank - 1 && v[L.rank - 1]) s.peer_recv[0] = v[L.rank - 1]->recv;
+    if (L.rank < L.nranks - 1 && (int)v.size() > L.rank + 1 && v[L.rank + 1]) s.peer_recv[1] = v[L.rank + 1]->recv;
+  }
+  const bool lo_nb = L.rank > 0, hi_nb = L.rank < L.nranks - 1;
+  if ((lo_nb && !s.peer_recv[0]) || (hi_nb && !s.peer_recv[1]))
+    return fail(STENCIL_E_INVALID, "stencil_run: a neighbour's receive area is unknown (every rank's plan must exist)");
+  const int64_t G = L.ghost, local_n = L.loc_hi - L.loc_lo;
+  const size_t chunk = (size_t)G * s.line_bytes;
+  const size_t pitch = (size_t)local_n * s.line_bytes;
+  const bool listed = s.rows_dev != nullptr && k >= 1 && (size_t)(2 * (k - 1) + 1) < s.row_span.size();
+  auto nrows = [&](int b) { return listed ? (size_t)s.row_span[2 * (k - 1) + b].second : (size_t)s.n_outer; };
+  auto rows = [&](int b) -> const int* { return listed ? s.rows_dev + s.row_span[2 * (k - 1) + b].first : nullptr; };
+  const int slot = (int)(k & 1);
+  auto area = [&](char* base, int side, int b) { return base + ((size_t)(slot * 2 + side) * 2 + b) * s.recv_halo; };
+  auto at = [&](int b, int64_t idx) { return static_cast<char*>(bufs[b]) + (size_t)idx * s.line_bytes; };
+  const int own0 = (int)(L.own_lo - L.loc_lo), own1 = (int)(L.own_hi - L.loc_lo);
+  const int seq = (int)(s.runs * (int64_t)(s.lay.n_blocks + 1) + k);
+  const int blocks = halo_blocks();
+  HaloCopyArgs snd{};
+  HaloSignal sig{};
+  for (int b = 0; b < 2; ++b) {
+    if (nrows(b) == 0) continue;
+    // I am my lower neighbour's upper neighbour (its side 1), and my upper neighbour's side 0
+    if (lo_nb) snd.reg[snd.n++] = HaloRegion{area(s.peer_recv[0], 1, b), at(b, own0), chunk, pitch, chunk, nrows(b), rows(b), nullptr};
+    if (hi_nb) snd.reg[snd.n++] = HaloRegion{area(s.peer_recv[1], 0, b), at(b, own1 - G), chunk, pitch, chunk, nrows(b), rows(b), nullptr};
+  }
+  if (s.emulate) {  // self-loop projection: publish exactly the flags this rank waits for
+    if (lo_nb) sig.flag[sig.n++] = reinterpret_cast<int*>(s.recv + s.flag_off) + 0;
+    if (hi_nb) sig.flag[sig.n++] = reinterpret_cast<int*>(s.recv + s.flag_off) + 1;
+  } else {
+    if (lo_nb) sig.flag[sig.n++] = reinterpret_cast<int*>(s.peer_recv[0] + s.flag_off) + 1;
+    if (hi_nb) sig.flag[sig.n++] = reinterpret_cast<int*>(s.peer_recv[1] + s.flag_off) + 0;
+  }
+  sig.done = reinterpret_cast<unsigned int*>(s.recv + s.flag_off + 64);
+  sig.done_base = s.done_count;
+  sig.seq = seq;
+  s.done_count += (unsigned int)blocks;
+  cudaError_t e = launch_halo_send(snd, sig, blocks, stream);
+  if (e != cudaSuccess) return fail(STENCIL_E_CUDA, std::string("stencil_run: halo send: ") + cudaGetErrorString(e));
+  HaloCopyArgs rcv{};
+  HaloWait w{};
+  for (int b = 0; b < 2; ++b) {
+    if (nrows(b) == 0) continue;
+    if (lo_nb) rcv.reg[rcv.n++] = HaloRegion{at(b, own0 - G), area(s.recv, 0, b), pitch, chunk, chunk, nrows(b), nullptr, rows(b)};
+    if (hi_nb) rcv.reg[rcv.n++] = HaloRegion{at(b, own1), area(s.recv, 1, b), pitch, chunk, chunk, nrows(b), nullptr, rows(b)};
+  }
+  if (lo_nb) w.flag[w.n++] = reinterpret_cast<const int*>(s.recv + s.flag_off) + 0;
+  if (hi_nb) w.flag[w.n++] = reinterpret_cast<const int*>(s.recv + s.flag_off) + 1;
+  w.seq = seq;
+  e = launch_halo_recv(rcv, w, blocks, stream);
+  if (e != cudaSuccess) return fail(STENCIL_E_CUDA, std::string("stencil_run: halo receive: ") + cudaGetErrorString(e));
+  return STENCIL_OK;
+}
+
 static stencil_status ghost_hook(void* ctx, int64_t k, void* const* bufs, void* stream) {
   DistState& s = *static_cast<DistState*>(ctx);
   if (s.lay.nranks <= 1 || (s.emulate && !s.emulate_copies)) return STENCIL_OK;
+  if (s.p2p) return exchange_p2p(s, k, bufs, static_cast<cudaStream_t>(stream));
   return exchange(s, k, bufs, static_cast<cudaStream_t>(stream));
 }
 
@@ -400,7 +519,9 @@ stencil_status run_dist(Plan& p, const void* const* in, void* const* out, void* 
   lp->pre_launch_ctx = &s;
   // the local plan copies in -> out and runs the global launch table over the slab, exchanging
   // the ghost planes before every launch but the first
-  return run_plan(*lp, in, out, stream);
+  const stencil_status st = run_plan(*lp, in, out, stream);
+  if (st == STENCIL_OK) ++s.runs;
+  return st;
 }
 
 }  // namespace hexs
@@ -506,8 +627,14 @@ stencil_status stencil_plan_dist(stencil_plan_t* out, stencil_desc_t global_desc
   // communicator, no exchanges (the ghost planes keep their initial values, so results are not
   // the global ones); it measures a rank's compute for scaling projections on a single GPU
   s->emulate = std::getenv("HEXS_DIST_EMULATE") && std::atoi(std::getenv("HEXS_DIST_EMULATE")) != 0;
-  s->emulate_copies = s->emulate && std::atoi(std::getenv("HEXS_DIST_EMULATE")) == 2;
-  if (!s->emulate) {  // (also for one rank: the same NCCL bootstrap path, no exchange ever runs)
+  // =2: plus the NCCL path's halo copies (a device-local copy as the wire); =3: plus the
+  // device-initiated path's kernels, the rank's own receive area standing in for its neighbours'
+  const int emu_mode = s->emulate ? std::atoi(std::getenv("HEXS_DIST_EMULATE")) : 0;
+  s->emulate_copies = emu_mode >= 2;
+  // HEXS_DIST_LOOPBACK=1: the ranks are plans of ONE process on one device (no communicator; the
+  // device-initiated exchange between them) -- the single-GPU test of the multi-rank protocol
+  s->loopback = !s->emulate && std::getenv("HEXS_DIST_LOOPBACK") && std::atoi(std::getenv("HEXS_DIST_LOOPBACK")) != 0;
+  if (!s->emulate && !s->loopback) {  // (also for one rank: the same NCCL bootstrap path, no exchange ever runs)
     NcclApi* a = nccl_api();
     if (!a) return fail(STENCIL_E_NCCL, "stencil_plan_dist: NCCL unavailable");
     ncclUniqueId id;
@@ -535,12 +662,71 @@ stencil_status stencil_plan_dist(stencil_plan_t* out, stencil_desc_t global_desc
   size_t ws = 0;
   for (auto& bp : s->bplans) ws = std::max(ws, bp.second->ws_bytes);
   s->local_ws = (ws + 255) / 256 * 256;
-  // strided partitions: staging for both buffers' 2 send + 2 receive halos
-  s->stage_bytes = s->n_outer > 1 && nranks > 1 ? 8 * (size_t)L.ghost * s->line_bytes * (size_t)s->n_outer : 0;
+  // Device-initiated exchange (default for nranks > 1; HEXS_DIST_P2P=0 keeps NCCL send/recv):
+  // a receive area in NCCL symmetric memory (ncclMemAlloc + ncclCommWindowRegister, collective),
+  // whose neighbours' views are the window's LSA pointers; loopback mode: cudaMalloc and the
+  // process-local registry.  Halo copies move 16-B units: chunk and pitch must be 16-B multiples.
+  {
+    const char* pe = std::getenv("HEXS_DIST_P2P");
+    const bool want = nranks > 1 && !(pe && std::atoi(pe) == 0) && (!s->emulate || emu_mode == 3);
+    const size_t chunk = (size_t)L.ghost * s->line_bytes;
+    const size_t pitch = (size_t)(L.loc_hi - L.loc_lo) * s->line_bytes;
+    if (want && chunk % 16 == 0 && pitch % 16 == 0) {
+      s->recv_halo = (chunk * (size_t)s->n_outer + 255) / 256 * 256;
+      s->flag_off = 8 * s->recv_halo;
+      s->recv_bytes = s->flag_off + 256;
+      if (emu_mode == 3) {  // self-loop: measures the send / wait / scatter kernels of one rank
+        void* r = nullptr;
+        if (cudaMalloc(&r, s->recv_bytes) != cudaSuccess || cudaMemset(r, 0, s->recv_bytes) != cudaSuccess)
+          return fail(STENCIL_E_OOM, "stencil_plan_dist: emulated receive area");
+        s->recv = static_cast<char*>(r);
+        s->loopback = true;  // (freed with cudaFree; no registry entry: group stays empty)
+        s->peer_recv[0] = s->peer_recv[1] = s->recv;
+        s->p2p = true;
+      } else if (s->loopback) {
+        void* r = nullptr;
+        if (cudaMalloc(&r, s->recv_bytes) != cudaSuccess || cudaMemset(r, 0, s->recv_bytes) != cudaSuccess)
+          return fail(STENCIL_E_OOM, "stencil_plan_dist: loopback receive area");
+        s->recv = static_cast<char*>(r);
+        s->group.assign(static_cast<const char*>(nccl_unique_id), 128);
+        std::lock_guard<std::mutex> lk(g_loop_mu);
+        auto& v = g_loop[s->group];
+        if ((int)v.size() < nranks) v.resize(nranks, nullptr);
+        v[rank] = s.get();
+        s->p2p = true;
+      } else if (NcclApi* a = nccl_api()) {
+        if (a->MemAlloc && a->WindowRegister && s->comm) {
+          void* r = nullptr;
+          if (a->MemAlloc(&r, s->recv_bytes) == ncclSuccess && r) {
+            s->recv = static_cast<char*>(r);
+            ncclWindow_t w = nullptr;
+            if (cudaMemset(r, 0, s->recv_bytes) == cudaSuccess &&
+                a->WindowRegister(static_cast<ncclComm_t>(s->comm), r, s->recv_bytes, &w, NCCL_WIN_COLL_SYMMETRIC) ==
+                    ncclSuccess &&
+                w) {
+              s->win = w;
+              void* pp = nullptr;
+              bool ok = true;
+              if (rank > 0) ok = ok && halo_peer_pointer(w, rank - 1, &pp, s->comm_stream) == cudaSuccess && pp;
+              if (ok && rank > 0) s->peer_recv[0] = static_cast<char*>(pp);
+              if (rank < nranks - 1) ok = ok && halo_peer_pointer(w, rank + 1, &pp, s->comm_stream) == cudaSuccess && pp;
+              if (ok && rank < nranks - 1) s->peer_recv[1] = static_cast<char*>(pp);
+              s->p2p = ok;
+            }
+            if (!s->p2p) s->release_p2p();  // fall back to ncclSend / ncclRecv
+          }
+        }
+      }
+    }
+    if (s->loopback && !s->p2p && nranks > 1)
+      return fail(STENCIL_E_UNSUPPORTED, "stencil_plan_dist: loopback mode needs 16-B aligned halos");
+  }
+  // strided partitions exchanged by NCCL send/recv: staging for both buffers' 2 send + 2 receive halos
+  s->stage_bytes = !s->p2p && s->n_outer > 1 && nranks > 1 ? 8 * (size_t)L.ghost * s->line_bytes * (size_t)s->n_outer : 0;
   // needed-state row lists: the hexagonal dimension 0 whole (its coordinate is the outer index
   // of the halo blocks), a classical dimension partitioned
   Plan* lp0 = s->bplans.empty() ? nullptr : s->bplans[0].second;
-  if (s->stage_bytes && lp0 && halo_rows_table(*lp0, pd, s->row_table, s->row_span)) {
+  if ((s->stage_bytes || (s->p2p && s->n_outer > 1)) && lp0 && halo_rows_table(*lp0, pd, s->row_table, s->row_span)) {
     s->rows_off = s->local_ws + s->stage_bytes;
     s->rows_bytes = (s->row_table.size() * sizeof(int) + 255) / 256 * 256;
   }

@@ -7,14 +7,16 @@
 // (profiles/round2/dist_y), several times their HBM time.
 #include <cstdint>
 
+#include <nccl.h>
+#include <nccl_device.h>
+
 #include "launch.h"
 
 namespace hexs {
 
 namespace {
 
-__global__ void __launch_bounds__(256) halo_copy_kernel(const __grid_constant__ HaloCopyArgs a) {
-  // flattened (region, row, 16-B column) index space
+__device__ __forceinline__ void copy_regions(const HaloCopyArgs& a) {
   int64_t total = 0;
 #pragma unroll 1
   for (int r = 0; r < a.n; ++r) total += (int64_t)a.reg[r].rows * (int64_t)(a.reg[r].width / 16);
@@ -36,7 +38,77 @@ __global__ void __launch_bounds__(256) halo_copy_kernel(const __grid_constant__ 
   }
 }
 
+// Sender: copy into peer memory, then the last block to finish publishes seq to the neighbours.
+__global__ void __launch_bounds__(256) halo_send_kernel(const __grid_constant__ HaloCopyArgs a,
+                                                        const __grid_constant__ HaloSignal sig) {
+  copy_regions(a);
+  __syncthreads();
+  if (threadIdx.x == 0) {
+    __threadfence_system();  // this block's peer stores before its completion count
+    const unsigned int prev = atomicAdd(sig.done, 1u);
+    if (prev == sig.done_base + gridDim.x - 1) {  // the last block: every block's stores are fenced
+      __threadfence_system();
+      for (int i = 0; i < sig.n; ++i)
+        asm volatile("st.release.sys.global.b32 [%0], %1;" ::"l"(sig.flag[i]), "r"(sig.seq) : "memory");
+    }
+  }
+}
+
+// Receiver: one warp waits for the neighbours' sequence numbers (a single small CTA, so a
+// co-scheduled peer kernel on the same device -- loopback mode -- always finds room); the
+// scatter runs after it in stream order.
+__global__ void __launch_bounds__(32) halo_wait_kernel(const __grid_constant__ HaloWait w) {
+  if (threadIdx.x == 0) {
+    for (int i = 0; i < w.n; ++i) {
+      while (true) {
+        int v;
+        asm volatile("ld.acquire.sys.global.b32 %0, [%1];" : "=r"(v) : "l"(w.flag[i]) : "memory");
+        if (v >= w.seq) break;
+        __nanosleep(256);
+      }
+    }
+    __threadfence_system();
+  }
+}
+
+__global__ void __launch_bounds__(256) halo_copy_kernel(const __grid_constant__ HaloCopyArgs a) {
+  copy_regions(a);
+}
+
+__global__ void peer_pointer_kernel(ncclWindow_t win, int peer, void** out) {
+  out[0] = ncclGetPeerPointer(win, 0, peer);
+}
+
 }  // namespace
+
+int halo_blocks() { return 4 * 148; }
+
+cudaError_t launch_halo_send(const HaloCopyArgs& a, const HaloSignal& sig, int blocks, cudaStream_t s) {
+  if (a.n > kMaxHaloRegions || sig.n > 2) return cudaErrorInvalidValue;
+  halo_send_kernel<<<blocks, 256, 0, s>>>(a, sig);
+  return cudaGetLastError();
+}
+
+cudaError_t launch_halo_recv(const HaloCopyArgs& a, const HaloWait& w, int blocks, cudaStream_t s) {
+  if (a.n > kMaxHaloRegions || w.n > 2) return cudaErrorInvalidValue;
+  halo_wait_kernel<<<1, 32, 0, s>>>(w);
+  cudaError_t e = cudaGetLastError();
+  if (e != cudaSuccess || a.n == 0) return e;
+  halo_copy_kernel<<<blocks, 256, 0, s>>>(a);
+  return cudaGetLastError();
+}
+
+cudaError_t halo_peer_pointer(void* win, int peer, void** out, cudaStream_t s) {
+  void** d = nullptr;
+  cudaError_t e = cudaMallocAsync(reinterpret_cast<void**>(&d), sizeof(void*), s);
+  if (e != cudaSuccess) return e;
+  peer_pointer_kernel<<<1, 1, 0, s>>>(static_cast<ncclWindow_t>(win), peer, d);
+  e = cudaGetLastError();
+  if (e == cudaSuccess) e = cudaMemcpyAsync(out, d, sizeof(void*), cudaMemcpyDeviceToHost, s);
+  if (e == cudaSuccess) e = cudaStreamSynchronize(s);
+  cudaFreeAsync(d, s);
+  return e;
+}
 
 cudaError_t launch_halo_copy(const HaloCopyArgs& a, cudaStream_t s) {
   if (a.n <= 0) return cudaSuccess;

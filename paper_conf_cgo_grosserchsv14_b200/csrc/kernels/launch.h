@@ -163,4 +163,27 @@ struct HaloCopyArgs {
 };
 cudaError_t launch_halo_copy(const HaloCopyArgs& a, cudaStream_t s);
 
+// Device-initiated halo exchange (kernels/halo.cu): the sender's kernel stores its halo lines
+// straight into the neighbours' receive staging (peer memory over NVLink: an NCCL symmetric
+// window's LSA pointers, or same-device pointers in loopback mode), and its last block publishes
+// `seq` into the neighbours' flags (system-scope release); the receiver's kernel waits for the
+// flags (acquire) and scatters its staging into its ghost lines.
+struct HaloSignal {
+  int n;                   // remote flags to publish
+  int* flag[2];            // neighbour flag words (peer memory)
+  unsigned int* done;      // this rank's block-completion counter (monotonic)
+  unsigned int done_base;  // counter value before this launch
+  int seq;
+};
+struct HaloWait {
+  int n;                   // local flags to wait for
+  const int* flag[2];
+  int seq;
+};
+cudaError_t launch_halo_send(const HaloCopyArgs& a, const HaloSignal& sig, int blocks, cudaStream_t s);
+cudaError_t launch_halo_recv(const HaloCopyArgs& a, const HaloWait& w, int blocks, cudaStream_t s);
+int halo_blocks();  // grid of the send / receive kernels (fixed, so the completion counter is exact)
+// NCCL symmetric window: the peer's view of offset 0 of window `win` (a device-side LSA lookup)
+cudaError_t halo_peer_pointer(void* win, int peer, void** out, cudaStream_t s);
+
 }  // namespace hexs

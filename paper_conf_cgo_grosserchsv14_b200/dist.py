@@ -173,13 +173,19 @@ class DistPlan:
     `global_ext`, over the ranks of `group` (one GPU each).  Collective constructor."""
 
     def __init__(self, kind: str, global_ext: Sequence[int], T: int, group=None, dtype="float32",
-                 part_dim: int = -1, **tile):
+                 part_dim: int = -1, rank: Optional[int] = None, nranks: Optional[int] = None,
+                 unique_id: Optional[bytes] = None, **tile):
+        """rank / nranks / unique_id: explicit (no process group) -- e.g. the loopback mode
+        (HEXS_DIST_LOOPBACK=1), where all ranks are plans of one process on one device and share
+        one id (any 128 bytes)."""
         self.kind = kind
         self.global_ext = tuple(int(e) for e in global_ext)
         self.T = int(T)
         self.group = group
         self.rank = dist.get_rank(group) if dist.is_initialized() else 0
         self.nranks = dist.get_world_size(group) if dist.is_initialized() else 1
+        if rank is not None:
+            self.rank, self.nranks = int(rank), int(nranks)
         emu = os.environ.get("HEXS_DIST_EMULATE_RANK")  # "r/P": play rank r of P alone (projection)
         if emu:
             r, P = (int(x) for x in emu.split("/"))
@@ -187,9 +193,11 @@ class DistPlan:
             self.rank, self.nranks = r, P
         self._d = _desc(kind, self.global_ext, dtype)
         uid = (ctypes.c_char * 128)()
-        if self.rank == 0:
+        if unique_id is not None:
+            ctypes.memmove(uid, bytes(unique_id)[:128].ljust(128, b"\0"), 128)
+        elif self.rank == 0:
             check(lib().stencil_dist_unique_id(uid))
-        if self.nranks > 1 and not emu:
+        if self.nranks > 1 and not emu and unique_id is None:
             obj = [bytes(uid) if self.rank == 0 else None]
             dist.broadcast_object_list(obj, src=dist.get_global_rank(group, 0) if group is not None else 0,
                                        group=group)
@@ -233,8 +241,9 @@ class DistPlan:
             return
         if self._ws is None or self._ws.device != device:
             self._ws = torch.empty(n.value + 256, dtype=torch.uint8, device=device)
-        ptr = (self._ws.data_ptr() + 255) // 256 * 256
-        check(lib().stencil_plan_set_workspace(self._h, ctypes.c_void_p(ptr), n.value))
+            ptr = (self._ws.data_ptr() + 255) // 256 * 256
+            # (once per allocation: setting it uploads the halo row lists synchronously)
+            check(lib().stencil_plan_set_workspace(self._h, ctypes.c_void_p(ptr), n.value))
 
     def run(self, local: torch.Tensor, out: Optional[torch.Tensor] = None, stream=None) -> torch.Tensor:
         """Collective: T steps; `local` holds level 0 on every plane of the slab.  Returns the
