@@ -66,6 +66,7 @@ struct NcclApi {
   ncclResult_t (*MemFree)(void*) = nullptr;
   ncclResult_t (*WindowRegister)(ncclComm_t, void*, size_t, ncclWindow_t*, int) = nullptr;
   ncclResult_t (*WindowDeregister)(ncclComm_t, ncclWindow_t) = nullptr;
+  ncclResult_t (*AllReduce)(const void*, void*, size_t, ncclDataType_t, ncclRedOp_t, ncclComm_t, cudaStream_t) = nullptr;
   std::string error;
 };
 
@@ -101,6 +102,7 @@ NcclApi* nccl_api() {
   api.MemFree = reinterpret_cast<decltype(api.MemFree)>(sym("ncclMemFree"));
   api.WindowRegister = reinterpret_cast<decltype(api.WindowRegister)>(sym("ncclCommWindowRegister"));
   api.WindowDeregister = reinterpret_cast<decltype(api.WindowDeregister)>(sym("ncclCommWindowDeregister"));
+  api.AllReduce = reinterpret_cast<decltype(api.AllReduce)>(sym("ncclAllReduce"));
   if (!api.GetUniqueId || !api.CommInitRank || !api.CommDestroy || !api.GroupStart || !api.GroupEnd ||
       !api.Send || !api.Recv || !api.GetErrorString) {
     api.error = "libnccl.so.2 lacks a required symbol";
@@ -670,8 +672,7 @@ stencil_status stencil_plan_dist(stencil_plan_t* out, stencil_desc_t global_desc
     const char* pe = std::getenv("HEXS_DIST_P2P");
     const bool want = nranks > 1 && !(pe && std::atoi(pe) == 0) && (!s->emulate || emu_mode == 3);
     const size_t chunk = (size_t)L.ghost * s->line_bytes;
-    const size_t pitch = (size_t)(L.loc_hi - L.loc_lo) * s->line_bytes;
-    if (want && chunk % 16 == 0 && pitch % 16 == 0) {
+    if (want && s->line_bytes % 16 == 0) {  // (rank-independent: every chunk and pitch 16-B granular)
       s->recv_halo = (chunk * (size_t)s->n_outer + 255) / 256 * 256;
       s->flag_off = 8 * s->recv_halo;
       s->recv_bytes = s->flag_off + 256;
@@ -695,27 +696,43 @@ stencil_status stencil_plan_dist(stencil_plan_t* out, stencil_desc_t global_desc
         v[rank] = s.get();
         s->p2p = true;
       } else if (NcclApi* a = nccl_api()) {
-        if (a->MemAlloc && a->WindowRegister && s->comm) {
-          void* r = nullptr;
-          if (a->MemAlloc(&r, s->recv_bytes) == ncclSuccess && r) {
-            s->recv = static_cast<char*>(r);
-            ncclWindow_t w = nullptr;
-            if (cudaMemset(r, 0, s->recv_bytes) == cudaSuccess &&
-                a->WindowRegister(static_cast<ncclComm_t>(s->comm), r, s->recv_bytes, &w, NCCL_WIN_COLL_SYMMETRIC) ==
-                    ncclSuccess &&
-                w) {
-              s->win = w;
-              void* pp = nullptr;
-              bool ok = true;
-              if (rank > 0) ok = ok && halo_peer_pointer(w, rank - 1, &pp, s->comm_stream) == cudaSuccess && pp;
-              if (ok && rank > 0) s->peer_recv[0] = static_cast<char*>(pp);
-              if (rank < nranks - 1) ok = ok && halo_peer_pointer(w, rank + 1, &pp, s->comm_stream) == cudaSuccess && pp;
-              if (ok && rank < nranks - 1) s->peer_recv[1] = static_cast<char*>(pp);
-              s->p2p = ok;
-            }
-            if (!s->p2p) s->release_p2p();  // fall back to ncclSend / ncclRecv
+        // every rank must take the same path (the window registration is collective): each step's
+        // local outcome is min-reduced over the communicator before the next
+        auto all_ok = [&](int ok) {
+          if (!s->comm || !a->AllReduce) return false;
+          int* dv = nullptr;
+          if (cudaMalloc(reinterpret_cast<void**>(&dv), sizeof(int)) != cudaSuccess) return false;
+          bool good = cudaMemcpy(dv, &ok, sizeof(int), cudaMemcpyHostToDevice) == cudaSuccess &&
+                      a->AllReduce(dv, dv, 1, ncclInt32, ncclMin, static_cast<ncclComm_t>(s->comm), s->comm_stream) ==
+                          ncclSuccess &&
+                      cudaStreamSynchronize(s->comm_stream) == cudaSuccess &&
+                      cudaMemcpy(&ok, dv, sizeof(int), cudaMemcpyDeviceToHost) == cudaSuccess;
+          cudaFree(dv);
+          return good && ok == 1;
+        };
+        void* r = nullptr;
+        const bool have = a->MemAlloc && a->WindowRegister && a->WindowDeregister && a->MemFree;
+        bool ok = have && a->MemAlloc(&r, s->recv_bytes) == ncclSuccess && r &&
+                  cudaMemset(r, 0, s->recv_bytes) == cudaSuccess;
+        if (r) s->recv = static_cast<char*>(r);
+        if (all_ok(ok ? 1 : 0)) {
+          ncclWindow_t w = nullptr;
+          ok = a->WindowRegister(static_cast<ncclComm_t>(s->comm), r, s->recv_bytes, &w, NCCL_WIN_COLL_SYMMETRIC) ==
+                   ncclSuccess &&
+               w;
+          if (w) s->win = w;
+          void* pp = nullptr;
+          if (ok && rank > 0) {
+            ok = halo_peer_pointer(w, rank - 1, &pp, s->comm_stream) == cudaSuccess && pp;
+            s->peer_recv[0] = static_cast<char*>(pp);
           }
+          if (ok && rank < nranks - 1) {
+            ok = halo_peer_pointer(w, rank + 1, &pp, s->comm_stream) == cudaSuccess && pp;
+            s->peer_recv[1] = static_cast<char*>(pp);
+          }
+          s->p2p = all_ok(ok ? 1 : 0);
         }
+        if (!s->p2p) s->release_p2p();  // fall back to ncclSend / ncclRecv
       }
     }
     if (s->loopback && !s->p2p && nranks > 1)
