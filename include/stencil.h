@@ -181,7 +181,19 @@ typedef struct {
   int32_t h;              /* hexagon half-height the time block is a multiple of             */
   double ghost_fraction;  /* (local - owned) / owned indices: the redundant work             */
   int64_t launches_per_run; /* phase-kernel launches of one stencil_run (stencil_dist_info) */
+  int32_t exchange;       /* stencil_dist_info: STENCIL_EXCHANGE_* the halos travel by          */
 } stencil_dist_info_t;
+
+enum {
+  STENCIL_EXCHANGE_NONE = 0,   /* one rank, or an emulated rank without halo traffic                */
+  STENCIL_EXCHANGE_NCCL = 1,   /* ncclSend / ncclRecv of packed halos on an internal stream         */
+  STENCIL_EXCHANGE_P2P = 2,    /* device-initiated: a send kernel stores the halo lines into the
+                                  neighbours' receive areas (NCCL symmetric window, LSA pointers)
+                                  and publishes a sequence number; a wait kernel acquires theirs   */
+  STENCIL_EXCHANGE_FUSED = 3   /* as P2P, but the 3D tile-wavefront phase kernel itself stores its
+                                  send-zone lines into the neighbours' mirrors while it computes
+                                  (y slabs of >= 2G lines): the transfer overlaps the launch       */
+};
 
 /* Rank 0: a fresh NCCL unique id (128 bytes) for stencil_plan_dist; broadcast it to the other
  * ranks (e.g. with torch.distributed).  STENCIL_E_NCCL if NCCL cannot be loaded. */

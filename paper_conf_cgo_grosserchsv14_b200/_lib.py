@@ -67,7 +67,9 @@ class DistInfo(ctypes.Structure):
                 ("own_lo", ctypes.c_int64), ("own_hi", ctypes.c_int64), ("loc_lo", ctypes.c_int64),
                 ("loc_hi", ctypes.c_int64), ("ghost", ctypes.c_int64), ("time_block", ctypes.c_int64),
                 ("n_blocks", ctypes.c_int64), ("h", ctypes.c_int32), ("ghost_fraction", ctypes.c_double),
-                ("launches_per_run", ctypes.c_int64)]
+                ("launches_per_run", ctypes.c_int64), ("exchange", ctypes.c_int32)]
+
+EXCHANGES = {0: "none", 1: "nccl", 2: "p2p", 3: "fused"}
 
 
 class TileEval(ctypes.Structure):

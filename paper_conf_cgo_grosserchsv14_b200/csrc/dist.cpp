@@ -148,6 +148,10 @@ struct DistState {
   // rank owns a receive area [slot k%2][side: from lower, from upper][buffer] x halo bytes + two
   // flags + a block counter; the sender's kernel stores straight into the neighbour's area.
   bool p2p = false, loopback = false;
+  // fused: the 3D tile-wavefront kernel itself stores its send-zone lines into the neighbours'
+  // mirrors while it computes (the transfer overlaps the launch); the boundary keeps only two
+  // flag handshakes and a local scatter
+  bool fused = false;
   char* recv = nullptr;
   size_t recv_bytes = 0, recv_halo = 0, flag_off = 0;
   void* win = nullptr;                      // ncclWindow_t of `recv`
@@ -499,9 +503,96 @@ static stencil_status exchange_p2p(DistState& s, int64_t k, void* const* bufs, c
   return STENCIL_OK;
 }
 
+// The fused exchange at the boundary before launch k.  Receive-area layout: mirror [side: from
+// lower, from upper][buffer parity][z][G lines][x] (each side's zone of the neighbour's state),
+// then the flags sent_from[lower, upper], scattered_from[lower, upper].
+//   k = 0: (after the previous run's last boundary has been consumed) seed the neighbours'
+//          mirrors with my send zones of both buffers;
+//   k > 0: my launch k-1 has stored into their mirrors: signal "sent", wait for theirs, scatter
+//          my mirror's needed rows into my ghost lines, signal "scattered", wait for theirs (they
+//          no longer read the mirrors my launch k will write).
+static void resolve_loop_peers(DistState& s) {
+  const DistLayout& L = s.lay;
+  if (!s.loopback || s.emulate) return;  // loopback: the neighbours are plans of this process
+  std::lock_guard<std::mutex> lk(g_loop_mu);
+  auto& v = g_loop[s.group];
+  if (L.rank > 0 && !s.peer_recv[0] && (int)v.size() > L.rank - 1 && v[L.rank - 1]) s.peer_recv[0] = v[L.rank - 1]->recv;
+  if (L.rank < L.nranks - 1 && !s.peer_recv[1] && (int)v.size() > L.rank + 1 && v[L.rank + 1])
+    s.peer_recv[1] = v[L.rank + 1]->recv;
+}
+
+static stencil_status exchange_fused(DistState& s, int64_t k, void* const* bufs, cudaStream_t stream) {
+  const DistLayout& L = s.lay;
+  resolve_loop_peers(s);
+  const bool lo_nb = L.rank > 0, hi_nb = L.rank < L.nranks - 1;
+  if ((lo_nb && !s.peer_recv[0]) || (hi_nb && !s.peer_recv[1]))
+    return fail(STENCIL_E_INVALID, "stencil_run: a neighbour's receive area is unknown (every rank's plan must exist)");
+  const int64_t G = L.ghost, local_n = L.loc_hi - L.loc_lo;
+  const size_t chunk = (size_t)G * s.line_bytes, pitch = (size_t)local_n * s.line_bytes;
+  const size_t M = chunk * (size_t)s.n_outer;  // one parity of one side's mirror
+  auto mirror = [&](char* base, int side, int b) { return base + ((size_t)side * 2 + b) * M; };
+  auto flags = [&](char* base) { return reinterpret_cast<int*>(base + s.flag_off); };
+  auto at = [&](int b, int64_t idx) { return static_cast<char*>(bufs[b]) + (size_t)idx * s.line_bytes; };
+  const int own0 = (int)(L.own_lo - L.loc_lo), own1 = (int)(L.own_hi - L.loc_lo);
+  const int seq = (int)(s.runs * (int64_t)(s.lay.n_blocks + 1) + k);
+  const int blocks = halo_blocks();
+  // flag word `idx` of my neighbour on side `nb_side` that refers to me (self-loop projection:
+  // the word of mine I will wait on)
+  auto remote = [&](int nb_side, int idx_base) -> int* {
+    if (s.emulate) return flags(s.recv) + idx_base + nb_side;
+    return flags(s.peer_recv[nb_side]) + idx_base + (1 - nb_side);
+  };
+  auto wait = [&](int idx_base, int sq) -> cudaError_t {
+    HaloCopyArgs none{};
+    HaloWait w{};
+    if (lo_nb) w.flag[w.n++] = flags(s.recv) + idx_base + 0;
+    if (hi_nb) w.flag[w.n++] = flags(s.recv) + idx_base + 1;
+    w.seq = sq;
+    return launch_halo_recv(none, w, blocks, stream);
+  };
+  auto signal = [&](int idx_base) -> cudaError_t {
+    int* f[2];
+    int n = 0;
+    if (lo_nb) f[n++] = remote(0, idx_base);
+    if (hi_nb) f[n++] = remote(1, idx_base);
+    return launch_halo_signal(n, f, seq, stream);
+  };
+  cudaError_t e = cudaSuccess;
+  if (k == 0) {
+    if (s.runs > 0) e = wait(2, seq - 2);  // the neighbours scattered the previous run's last data
+    HaloCopyArgs cp{};
+    for (int b = 0; b < 2 && e == cudaSuccess; ++b) {
+      char* lo_dst = s.emulate ? mirror(s.recv, 0, b) : (lo_nb ? mirror(s.peer_recv[0], 1, b) : nullptr);
+      char* hi_dst = s.emulate ? mirror(s.recv, 1, b) : (hi_nb ? mirror(s.peer_recv[1], 0, b) : nullptr);
+      if (lo_nb) cp.reg[cp.n++] = HaloRegion{lo_dst, at(b, own0), chunk, pitch, chunk, (size_t)s.n_outer, nullptr, nullptr};
+      if (hi_nb) cp.reg[cp.n++] = HaloRegion{hi_dst, at(b, own1 - G), chunk, pitch, chunk, (size_t)s.n_outer, nullptr, nullptr};
+    }
+    if (e == cudaSuccess) e = launch_halo_copy(cp, stream);
+  } else {
+    const bool listed = s.rows_dev != nullptr && (size_t)(2 * (k - 1) + 1) < s.row_span.size();
+    auto nrows = [&](int b) { return listed ? (size_t)s.row_span[2 * (k - 1) + b].second : (size_t)s.n_outer; };
+    auto rows = [&](int b) -> const int* { return listed ? s.rows_dev + s.row_span[2 * (k - 1) + b].first : nullptr; };
+    e = signal(0);
+    if (e == cudaSuccess) e = wait(0, seq);
+    HaloCopyArgs sc{};
+    for (int b = 0; b < 2; ++b) {
+      if (nrows(b) == 0) continue;
+      if (lo_nb) sc.reg[sc.n++] = HaloRegion{at(b, own0 - G), mirror(s.recv, 0, b), pitch, chunk, chunk, nrows(b), rows(b), rows(b)};
+      if (hi_nb) sc.reg[sc.n++] = HaloRegion{at(b, own1), mirror(s.recv, 1, b), pitch, chunk, chunk, nrows(b), rows(b), rows(b)};
+    }
+    if (e == cudaSuccess) e = launch_halo_copy(sc, stream);
+    if (e == cudaSuccess) e = signal(2);
+    if (e == cudaSuccess) e = wait(2, seq);
+  }
+  if (e != cudaSuccess) return fail(STENCIL_E_CUDA, std::string("stencil_run: fused halo exchange: ") + cudaGetErrorString(e));
+  return STENCIL_OK;
+}
+
 static stencil_status ghost_hook(void* ctx, int64_t k, void* const* bufs, void* stream) {
   DistState& s = *static_cast<DistState*>(ctx);
   if (s.lay.nranks <= 1 || (s.emulate && !s.emulate_copies)) return STENCIL_OK;
+  if (s.fused) return exchange_fused(s, k, bufs, static_cast<cudaStream_t>(stream));
+  if (k == 0) return STENCIL_OK;  // (the other paths exchange before launches k >= 1 only)
   if (s.p2p) return exchange_p2p(s, k, bufs, static_cast<cudaStream_t>(stream));
   return exchange(s, k, bufs, static_cast<cudaStream_t>(stream));
 }
@@ -519,6 +610,20 @@ stencil_status run_dist(Plan& p, const void* const* in, void* const* out, void* 
   if (!lp) return STENCIL_OK;
   lp->pre_launch = ghost_hook;
   lp->pre_launch_ctx = &s;
+  lp->mir[0] = lp->mir[1] = nullptr;
+  lp->mir_G = 0;
+  resolve_loop_peers(s);
+  if (s.fused && s.lay.nranks > 1) {  // the phase kernel mirrors its send zones (local lines)
+    const size_t M = (size_t)s.lay.ghost * s.line_bytes * (size_t)s.n_outer;
+    const bool lo_nb = s.lay.rank > 0, hi_nb = s.lay.rank < s.lay.nranks - 1;
+    char* lo_base = s.emulate ? s.recv : s.peer_recv[0];
+    char* hi_base = s.emulate ? s.recv : s.peer_recv[1];
+    if (lo_nb && lo_base) lp->mir[0] = lo_base + (s.emulate ? 0 : 2 * M);   // the lower neighbour's side 1
+    if (hi_nb && hi_base) lp->mir[1] = hi_base + (s.emulate ? 2 * M : 0);   // the upper neighbour's side 0
+    lp->mir_y0[0] = (int)(s.lay.own_lo - s.lay.loc_lo);
+    lp->mir_y0[1] = (int)(s.lay.own_hi - s.lay.loc_lo - s.lay.ghost);
+    lp->mir_G = (int)s.lay.ghost;
+  }
   // the local plan copies in -> out and runs the global launch table over the slab, exchanging
   // the ghost planes before every launch but the first
   const stencil_status st = run_plan(*lp, in, out, stream);
@@ -748,6 +853,13 @@ stencil_status stencil_plan_dist(stencil_plan_t* out, stencil_desc_t global_desc
     s->rows_bytes = (s->row_table.size() * sizeof(int) + 255) / 256 * 256;
   }
   p->ws_bytes = s->local_ws + s->stage_bytes + s->rows_bytes;
+  // fused halo stores: the 3D tile-wavefront kernel on y slabs of at least 2G lines (rank-
+  // independent test: the smallest slab), unless HEXS_DIST_FUSED=0
+  {
+    const char* fe = std::getenv("HEXS_DIST_FUSED");
+    s->fused = s->p2p && lp0 && lp0->executor == EXEC_FAST3D && pd == 1 && lp0->hd == 0 &&
+               d->ext[pd] / nranks >= 2 * L.ghost && !(fe && std::atoi(fe) == 0);
+  }
   p->dist = s.release();
   *out = reinterpret_cast<stencil_plan_t>(p);
   return STENCIL_OK;
@@ -827,6 +939,10 @@ stencil_status stencil_dist_info(stencil_plan_t plan, stencil_dist_info_t* info)
     launches += bp->executor == EXEC_NAIVE ? bp->tau_levels : (int64_t)bp->launches.size();
   }
   o.launches_per_run = launches;
+  o.exchange = L.nranks <= 1 || (s.emulate && !s.emulate_copies) ? STENCIL_EXCHANGE_NONE
+               : s.fused                                        ? STENCIL_EXCHANGE_FUSED
+               : s.p2p                                          ? STENCIL_EXCHANGE_P2P
+                                                                : STENCIL_EXCHANGE_NCCL;
   *info = o;
   return STENCIL_OK;
 }

@@ -104,6 +104,11 @@ struct Plan {
   // slab mode: the per-launch ghost exchange); nullptr = none
   stencil_status (*pre_launch)(void* ctx, int64_t k, void* const* bufs, void* stream) = nullptr;
   void* pre_launch_ctx = nullptr;
+  // fused halo stores of the 3D tile-wavefront kernel (slab mode, set per run by dist.cpp):
+  // neighbour s's mirror base, the first local line of the zone it mirrors, the zone width
+  void* mir[2] = {nullptr, nullptr};
+  int mir_y0[2] = {0, 0};
+  int mir_G = 0;
   std::vector<int32_t> lo, hi;  // hexagon rows per level a
   std::vector<Launch> launches;
   int executor = EXEC_GENERIC;

@@ -71,6 +71,12 @@ __global__ void __launch_bounds__(32) halo_wait_kernel(const __grid_constant__ H
   }
 }
 
+__global__ void halo_signal_kernel(int n, int* f0, int* f1, int seq) {
+  __threadfence_system();
+  if (n > 0) asm volatile("st.release.sys.global.b32 [%0], %1;" ::"l"(f0), "r"(seq) : "memory");
+  if (n > 1) asm volatile("st.release.sys.global.b32 [%0], %1;" ::"l"(f1), "r"(seq) : "memory");
+}
+
 __global__ void __launch_bounds__(256) halo_copy_kernel(const __grid_constant__ HaloCopyArgs a) {
   copy_regions(a);
 }
@@ -108,6 +114,13 @@ cudaError_t halo_peer_pointer(void* win, int peer, void** out, cudaStream_t s) {
   if (e == cudaSuccess) e = cudaStreamSynchronize(s);
   cudaFreeAsync(d, s);
   return e;
+}
+
+cudaError_t launch_halo_signal(int n, int* const* flags, int seq, cudaStream_t s) {
+  if (n <= 0) return cudaSuccess;
+  if (n > 2) return cudaErrorInvalidValue;
+  halo_signal_kernel<<<1, 1, 0, s>>>(n, flags[0], n > 1 ? flags[1] : nullptr, seq);
+  return cudaGetLastError();
 }
 
 cudaError_t launch_halo_copy(const HaloCopyArgs& a, cudaStream_t s) {

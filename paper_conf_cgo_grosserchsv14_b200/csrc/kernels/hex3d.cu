@@ -270,7 +270,9 @@ __device__ __forceinline__ void for_levels(F&& f, std::integer_sequence<int, As.
 
 // NY tile lines (y); ZS threads per (line, quad), each sweeping 1/ZS of a level's rows;
 // MINB CTAs per SM; plus one producer warp
-template <typename T, int KIND, int H, int W0, int NY, int MINB, int ZS>
+// MIR: the fused halo stores of the multi-GPU slab mode (a separate instantiation, so the
+// single-GPU kernel keeps its register budget)
+template <typename T, int KIND, int H, int W0, int NY, int MINB, int ZS, bool MIR>
 __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const __grid_constant__ Fast3DArgs g,
                                                                    const __grid_constant__ Maps mp) {
   using HX = Hex<H, W0>;
@@ -534,6 +536,21 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
           const uint32_t zsel = ((OMASK & zm_out) | (~OMASK & zm_non)) >> R0;
           // store pointer of row LO, advanced one plane per row (a predicated store per row)
           T* gp = static_cast<T*>(g.buf[(g.tau0 + A + 1) & 1]) + (i0 + R0) * plane + (int64_t)y * N2 + xb;
+          // fused halo stores: this thread's line in a neighbour's send zone (slab mode)
+          const int64_t mplane = (int64_t)g.mir_G * N2;
+          auto mir_at = [&](int s) -> T* {
+            if (!g.mir[s] || y < g.mir_y0[s] || y >= g.mir_y0[s] + g.mir_G) return nullptr;
+            return static_cast<T*>(g.mir[s]) + ((int64_t)((g.tau0 + A + 1) & 1) * N0 + (i0 + R0)) * mplane +
+                   (int64_t)(y - g.mir_y0[s]) * N2 + xb;
+          };
+          // (the two send zones are disjoint -- the slab mode fuses only slabs of >= 2G lines --
+          // so a line belongs to at most one neighbour's mirror)
+          T* mpp = nullptr;
+          if constexpr (MIR) {
+            mpp = mir_at(0);
+            if (!mpp) mpp = mir_at(1);
+          }
+          const bool mon = mpp != nullptr;  // (the pointer advances per row; the flag does not)
 
           const T* Pr[3] = {P[0], P[1], P[2]};
           auto adv = [&]() {
@@ -569,14 +586,21 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
               }
             }
             if ((zsel >> i) & 1u) {
-              if constexpr (sizeof(T) == 4) {
-                reinterpret_cast<float4*>(gp)[0] = make_float4(out[0], out[1], out[2], out[3]);
-              } else {
-                reinterpret_cast<double2*>(gp)[0] = make_double2(out[0], out[1]);
-                reinterpret_cast<double2*>(gp)[1] = make_double2(out[2], out[3]);
+              auto st4 = [&](T* d) {
+                if constexpr (sizeof(T) == 4) {
+                  reinterpret_cast<float4*>(d)[0] = make_float4(out[0], out[1], out[2], out[3]);
+                } else {
+                  reinterpret_cast<double2*>(d)[0] = make_double2(out[0], out[1]);
+                  reinterpret_cast<double2*>(d)[1] = make_double2(out[2], out[3]);
+                }
+              };
+              st4(gp);
+              if constexpr (MIR) {
+                if (mon) st4(mpp);
               }
             }
             gp += plane;
+            if constexpr (MIR) mpp += mplane;
           };
           if constexpr (KIND == K_STAR3D7 && HEXS_F3_UNROLL && ZS == 1) {
             // short per-point expression: the whole sweep unrolled and software-pipelined
@@ -681,13 +705,13 @@ static bool encode(CUtensorMap* map, void* base, const Fast3DArgs& a, uint32_t b
             CU_TENSOR_MAP_L2_PROMOTION_L2_128B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE) == CUDA_SUCCESS;
 }
 
-template <typename T, int KIND, int H, int W0, int NY, int MINB, int ZS>
+template <typename T, int KIND, int H, int W0, int NY, int MINB, int ZS, bool MIR>
 cudaError_t launch_t(const Fast3DArgs& a, cudaStream_t s) {
   using LY = Lay<T, Hex<H, W0>::Q, NY>;
   constexpr int NT = ZS * NY * NQ + 32;  // compute threads + the producer warp
   static DeviceMemo<int> memo;  // per device: smem opt-in + persistent grid size
   constexpr size_t smem = LY::SMEM;
-  auto kern = fast3d_kernel<T, KIND, H, W0, NY, MINB, ZS>;
+  auto kern = fast3d_kernel<T, KIND, H, W0, NY, MINB, ZS, MIR>;
   int grid = 0;
   cudaError_t e0 = memo.get(&grid, [&](int dev, int* gsz) {
     cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
@@ -731,7 +755,9 @@ HEXS_FAST3D_VARIANTS(HEXS_F3_SEL)
 using S3 = Sel3<HEXS_F3_VARIANT>;
 
 cudaError_t HEXS_F3_CAT(launch_fast3d_v, HEXS_F3_VARIANT)(const Fast3DArgs& a, cudaStream_t s) {
-  return fast3d::launch_t<S3::T, S3::KIND, S3::H, S3::W0, S3::NY, S3::MINB, S3::ZS>(a, s);
+  if (a.mir[0] || a.mir[1])
+    return fast3d::launch_t<S3::T, S3::KIND, S3::H, S3::W0, S3::NY, S3::MINB, S3::ZS, true>(a, s);
+  return fast3d::launch_t<S3::T, S3::KIND, S3::H, S3::W0, S3::NY, S3::MINB, S3::ZS, false>(a, s);
 }
 #ifdef HEXS_F3_TRACE
 extern "C" int HEXS_F3_CAT(hexs_f3_trace_v, HEXS_F3_VARIANT)(unsigned long long* host, int* counts, int reset) {

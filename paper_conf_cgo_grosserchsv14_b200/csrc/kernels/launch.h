@@ -99,6 +99,12 @@ struct Fast3DArgs {
   int* flags;                   // per tile completion flag, zeroed per launch
   unsigned long long* counter;  // work counter, zeroed per launch
   int32_t lo[kMaxH], hi[kMaxH];
+  // Fused halo stores (multi-GPU slab mode along y, csrc/dist.cpp): every global store of a line
+  // y in [mir_y0[s], mir_y0[s] + mir_G) is also written into neighbour s's mirror (peer memory),
+  // laid out [buffer parity][z][y - mir_y0[s]][x]; mir[s] = nullptr: none.
+  void* mir[2];
+  int mir_y0[2];
+  int mir_G;
 };
 cudaError_t launch_fast3d(int variant, const Fast3DArgs& a, int grid, cudaStream_t s);
 constexpr int kFast3DNX = 32;            // classical tile width along x of the 3D fast kernel
@@ -183,6 +189,9 @@ struct HaloWait {
 cudaError_t launch_halo_send(const HaloCopyArgs& a, const HaloSignal& sig, int blocks, cudaStream_t s);
 cudaError_t launch_halo_recv(const HaloCopyArgs& a, const HaloWait& w, int blocks, cudaStream_t s);
 int halo_blocks();  // grid of the send / receive kernels (fixed, so the completion counter is exact)
+// publish seq into up to 2 flag words (peer memory) after a system-scope fence: everything this
+// stream wrote before (e.g. a phase kernel's fused halo stores) is visible to the flags' readers
+cudaError_t launch_halo_signal(int n, int* const* flags, int seq, cudaStream_t s);
 // NCCL symmetric window: the peer's view of offset 0 of window `win` (a device-side LSA lookup)
 cudaError_t halo_peer_pointer(void* win, int peer, void** out, cudaStream_t s);
 

@@ -149,7 +149,7 @@ stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* 
                 "stencil_run: reset strip progress counters");
     int64_t launch_k = 0;
     for (const Launch& l : p.launches) {
-      if (p.pre_launch && launch_k > 0) {
+      if (p.pre_launch) {  // (k = 0 too: the slab mode's fused exchange seeds the mirrors)
         void* const bufs[2] = {buf[0], buf[1]};
         const stencil_status hs = p.pre_launch(p.pre_launch_ctx, launch_k, bufs, s);
         if (hs != STENCIL_OK) return hs;
@@ -284,6 +284,11 @@ stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* 
         }
         char* ws = static_cast<char*>(p.ws);
         a.flags = reinterpret_cast<int*>(ws + p.flag_off) + l.flag_first;
+        for (int q = 0; q < 2; ++q) {
+          a.mir[q] = p.mir[q];
+          a.mir_y0[q] = p.mir_y0[q];
+        }
+        a.mir_G = p.mir_G;
         a.counter = reinterpret_cast<unsigned long long*>(ws + p.counter_off) + l.counter_idx;
         HEXS_CUDA(launch_fast3d(p.variant, a, grid, s), "stencil_run: fast3d kernel launch");
       } else {

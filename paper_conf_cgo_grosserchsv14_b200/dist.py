@@ -211,6 +211,7 @@ class DistPlan:
         check(lib().stencil_dist_info(h, ctypes.byref(info)))
         self.layout = _layout_of(info, len(self.global_ext), self.global_ext)
         self.launches_per_run = int(info.launches_per_run)
+        self.exchange = _lib.EXCHANGES.get(int(info.exchange), str(info.exchange))
         self._ws = None
         self.dtype = dtype
 
@@ -421,7 +422,7 @@ def bench_main(args, cfg, configs, metric, helpers):
                 "config": {"workload": cname + (f" weak-scaled to {gext[0]} planes over {world} GPUs"
                                                 if scaling == "weak" else f" over {world} GPUs"),
                            "kind": kind, "extents": list(gext), "T": T, "partition": f"dim {pd} slabs",
-                           "time_block": lay.time_block, "ghost_indices": lay.ghost,
+                           "time_block": lay.time_block, "ghost_indices": lay.ghost, "halo_exchange": dp.exchange,
                            "ghost_fraction": lay.ghost_fraction, "local_extents": list(lay.local_ext),
                            "l2": "inputs larger than L2 (per-rank slab > 126 MB)"},
                 "roofline": roof,

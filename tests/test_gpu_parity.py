@@ -286,10 +286,12 @@ def test_linear_stencils(case, executor, dtype):
     assert_bitexact(out.cpu().numpy(), oracle.linear(g, offs, coefs, T), f"linear case {case} {executor}")
 
 
-@pytest.mark.parametrize("kind,ext,T,P,pd", [("star3d7", (40, 64, 72), 23, 2, 1), ("star3d7", (33, 70, 132), 17, 3, 1),
-                                             ("star3d7", (60, 40, 64), 19, 2, 0), ("star2d5", (300, 512), 29, 3, -1),
-                                             ("box3d27", (30, 52, 64), 13, 2, 1)])
-def test_dist_loopback_device_initiated_halo(kind, ext, T, P, pd):
+@pytest.mark.parametrize("kind,ext,T,P,pd,fused,mode", [
+    ("star3d7", (40, 64, 72), 23, 2, 1, "1", "fused"), ("star3d7", (33, 70, 132), 17, 3, 1, "1", "fused"),
+    ("star3d7", (33, 70, 132), 17, 3, 1, "0", "p2p"), ("star3d7", (60, 40, 64), 19, 2, 0, "1", "p2p"),
+    ("star2d5", (300, 512), 29, 3, -1, "1", "p2p"), ("box3d27", (30, 52, 64), 13, 2, 1, "1", "fused"),
+    ("gradient3d", (21, 80, 68), 9, 4, 1, "1", "fused")])
+def test_dist_loopback_device_initiated_halo(kind, ext, T, P, pd, fused, mode):
     """The device-initiated halo exchange (csrc/dist.cpp exchange_p2p, kernels/halo.cu) between P
     ranks that are plans of one process on this GPU (HEXS_DIST_LOOPBACK=1; tools/loop_check.py,
     in a subprocess with eager module loading): every rank's send kernel stores its halo lines
@@ -302,7 +304,8 @@ def test_dist_loopback_device_initiated_halo(kind, ext, T, P, pd):
     import sys
 
     root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
-    env = dict(os.environ, CUDA_MODULE_LOADING="EAGER")
+    env = dict(os.environ, CUDA_MODULE_LOADING="EAGER", HEXS_DIST_FUSED=fused)
     r = subprocess.run([sys.executable, os.path.join(root, "tools", "loop_check.py"), kind, ",".join(map(str, ext)),
                         str(T), str(P), str(pd)], env=env, capture_output=True, text=True, timeout=180)
     assert r.returncode == 0 and r.stdout.startswith("OK"), r.stdout + r.stderr[-2000:]
+    assert f"exchange={mode}" in r.stdout, r.stdout

@@ -40,7 +40,7 @@ def main(kind, ext, T, P, pd):
             print(f"MISMATCH run {it}: {len(bad)} values, first {tuple(bad[0])}", flush=True)
             return 1
     print(f"OK {kind} {ext} T={T} P={P} part_dim={plans[0].layout.part_dim} "
-          f"launches={plans[0].launches_per_run}", flush=True)
+          f"launches={plans[0].launches_per_run} exchange={plans[0].exchange}", flush=True)
     return 0
 
 
