@@ -192,7 +192,8 @@ enum {
                                   and publishes a sequence number; a wait kernel acquires theirs   */
   STENCIL_EXCHANGE_FUSED = 3   /* as P2P, but the 3D tile-wavefront phase kernel itself stores its
                                   send-zone lines into the neighbours' mirrors while it computes
-                                  (y slabs of >= 2G lines): the transfer overlaps the launch       */
+                                  (y slabs of >= 2G lines; opt-in, environment HEXS_DIST_FUSED=1):
+                                  the transfer overlaps the launch                                 */
 };
 
 /* Rank 0: a fresh NCCL unique id (128 bytes) for stencil_plan_dist; broadcast it to the other

@@ -613,7 +613,8 @@ stencil_status run_dist(Plan& p, const void* const* in, void* const* out, void* 
   lp->mir[0] = lp->mir[1] = nullptr;
   lp->mir_G = 0;
   resolve_loop_peers(s);
-  if (s.fused && s.lay.nranks > 1) {  // the phase kernel mirrors its send zones (local lines)
+  static const bool no_store = std::getenv("HEXS_DIST_FUSED_NOSTORE") && std::atoi(std::getenv("HEXS_DIST_FUSED_NOSTORE"));
+  if (s.fused && s.lay.nranks > 1 && !no_store) {  // the phase kernel mirrors its send zones (local lines)
     const size_t M = (size_t)s.lay.ghost * s.line_bytes * (size_t)s.n_outer;
     const bool lo_nb = s.lay.rank > 0, hi_nb = s.lay.rank < s.lay.nranks - 1;
     char* lo_base = s.emulate ? s.recv : s.peer_recv[0];
@@ -623,6 +624,9 @@ stencil_status run_dist(Plan& p, const void* const* in, void* const* out, void* 
     lp->mir_y0[0] = (int)(s.lay.own_lo - s.lay.loc_lo);
     lp->mir_y0[1] = (int)(s.lay.own_hi - s.lay.loc_lo - s.lay.ghost);
     lp->mir_G = (int)s.lay.ghost;
+    // (HEXS_DIST_MIRFENCE=0: no system-scope fence -- measurement aid only)
+    static const char* mf = std::getenv("HEXS_DIST_MIRFENCE");
+    lp->mir_fence = mf ? std::atoi(mf) : 1;
   }
   // the local plan copies in -> out and runs the global launch table over the slab, exchanging
   // the ghost planes before every launch but the first
@@ -853,12 +857,14 @@ stencil_status stencil_plan_dist(stencil_plan_t* out, stencil_desc_t global_desc
     s->rows_bytes = (s->row_table.size() * sizeof(int) + 255) / 256 * 256;
   }
   p->ws_bytes = s->local_ws + s->stage_bytes + s->rows_bytes;
-  // fused halo stores: the 3D tile-wavefront kernel on y slabs of at least 2G lines (rank-
-  // independent test: the smallest slab), unless HEXS_DIST_FUSED=0
+  // fused halo stores (HEXS_DIST_FUSED=1, opt-in): the 3D tile-wavefront kernel on y slabs of at
+  // least 2G lines (rank-independent test: the smallest slab).  Measured: its
+  // mirror-storing instantiation runs ~15 % slower than the plain kernel, which eats the overlap
+  // it buys, so the separate device-initiated exchange stays the default
   {
     const char* fe = std::getenv("HEXS_DIST_FUSED");
     s->fused = s->p2p && lp0 && lp0->executor == EXEC_FAST3D && pd == 1 && lp0->hd == 0 &&
-               d->ext[pd] / nranks >= 2 * L.ghost && !(fe && std::atoi(fe) == 0);
+               d->ext[pd] / nranks >= 2 * L.ghost && fe && std::atoi(fe) != 0;
   }
   p->dist = s.release();
   *out = reinterpret_cast<stencil_plan_t>(p);

@@ -109,6 +109,7 @@ struct Plan {
   void* mir[2] = {nullptr, nullptr};
   int mir_y0[2] = {0, 0};
   int mir_G = 0;
+  int mir_fence = 1;
   std::vector<int32_t> lo, hi;  // hexagon rows per level a
   std::vector<Launch> launches;
   int executor = EXEC_GENERIC;

@@ -492,6 +492,7 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
                       X0 - SIGMA * a_hi < 1 || X0 - SIGMA * a_lo + NX - 1 > N2 - 2;
     F3_TM(3);
 
+    bool mir_used = false;  // this thread stored into a neighbour's mirror during the tile
     for_levels(
         [&](auto ac) {
           constexpr int A = decltype(ac)::value;
@@ -536,21 +537,22 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
           const uint32_t zsel = ((OMASK & zm_out) | (~OMASK & zm_non)) >> R0;
           // store pointer of row LO, advanced one plane per row (a predicated store per row)
           T* gp = static_cast<T*>(g.buf[(g.tau0 + A + 1) & 1]) + (i0 + R0) * plane + (int64_t)y * N2 + xb;
-          // fused halo stores: this thread's line in a neighbour's send zone (slab mode)
-          const int64_t mplane = (int64_t)g.mir_G * N2;
-          auto mir_at = [&](int s) -> T* {
-            if (!g.mir[s] || y < g.mir_y0[s] || y >= g.mir_y0[s] + g.mir_G) return nullptr;
-            return static_cast<T*>(g.mir[s]) + ((int64_t)((g.tau0 + A + 1) & 1) * N0 + (i0 + R0)) * mplane +
-                   (int64_t)(y - g.mir_y0[s]) * N2 + xb;
-          };
-          // (the two send zones are disjoint -- the slab mode fuses only slabs of >= 2G lines --
-          // so a line belongs to at most one neighbour's mirror)
+          // fused halo stores (slab mode): a line of a neighbour's send zone is also stored into
+          // that neighbour's mirror [parity][z][y - zone start][x] (peer memory); the zones are
+          // disjoint (slabs of >= 2G lines), so a line has at most one mirror
           T* mpp = nullptr;
+          int64_t mplane = 0;
           if constexpr (MIR) {
-            mpp = mir_at(0);
-            if (!mpp) mpp = mir_at(1);
+            mplane = (int64_t)g.mir_G * N2;
+            const int side = (g.mir[0] && y >= g.mir_y0[0] && y < g.mir_y0[0] + g.mir_G)   ? 0
+                             : (g.mir[1] && y >= g.mir_y0[1] && y < g.mir_y0[1] + g.mir_G) ? 1
+                                                                                            : -1;
+            if (side >= 0)
+              mpp = static_cast<T*>(g.mir[side]) + ((int64_t)((g.tau0 + A + 1) & 1) * N0 + (i0 + R0)) * mplane +
+                    (int64_t)(y - g.mir_y0[side]) * N2 + xb;
           }
-          const bool mon = mpp != nullptr;  // (the pointer advances per row; the flag does not)
+          const bool mon = MIR && mpp != nullptr;  // (the pointer advances per row; the flag does not)
+          if constexpr (MIR) mir_used |= mon;
 
           const T* Pr[3] = {P[0], P[1], P[2]};
           auto adv = [&]() {
@@ -596,7 +598,17 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
               };
               st4(gp);
               if constexpr (MIR) {
-                if (mon) st4(mpp);
+                // the mirror is never read by this kernel: an asm store the compiler schedules
+                // freely (no ordering against the level buffers' shared loads)
+                if (mon) {
+                  if constexpr (sizeof(T) == 4) {
+                    asm volatile("st.global.v4.f32 [%0], {%1, %2, %3, %4};" ::"l"(mpp), "f"(out[0]), "f"(out[1]),
+                                 "f"(out[2]), "f"(out[3]));
+                  } else {
+                    asm volatile("st.global.v2.f64 [%0], {%1, %2};" ::"l"(mpp), "d"(out[0]), "d"(out[1]));
+                    asm volatile("st.global.v2.f64 [%0], {%1, %2};" ::"l"(mpp + 2), "d"(out[2]), "d"(out[3]));
+                  }
+                }
               }
             }
             gp += plane;
@@ -671,6 +683,12 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
           F3_TM(3);
         },
         std::make_integer_sequence<int, L>{});
+    if constexpr (MIR) {
+      // fused halo stores: the threads that wrote into a mirror fence at system scope before the
+      // barrier, so the tile's peer stores are ordered before its flag and a successor's later
+      // store to the same mirror place lands last
+      if (g.mir_fence && mir_used) __threadfence_system();
+    }
     named_barrier_sync(1, NC);  // every compute thread's stores of the tile are issued
     F3_TM(1);
     if (tid == 0) st_release(my_flag, 1);

@@ -105,6 +105,7 @@ struct Fast3DArgs {
   void* mir[2];
   int mir_y0[2];
   int mir_G;
+  int mir_fence;  // 1: each thread that stored into a mirror fences at system scope before the tile's flag
 };
 cudaError_t launch_fast3d(int variant, const Fast3DArgs& a, int grid, cudaStream_t s);
 constexpr int kFast3DNX = 32;            // classical tile width along x of the 3D fast kernel

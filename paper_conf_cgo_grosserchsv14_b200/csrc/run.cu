@@ -289,6 +289,7 @@ stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* 
           a.mir_y0[q] = p.mir_y0[q];
         }
         a.mir_G = p.mir_G;
+        a.mir_fence = p.mir_fence;
         a.counter = reinterpret_cast<unsigned long long*>(ws + p.counter_off) + l.counter_idx;
         HEXS_CUDA(launch_fast3d(p.variant, a, grid, s), "stencil_run: fast3d kernel launch");
       } else {
