@@ -39,6 +39,10 @@
 #ifndef HEXS_MERGE_ROWP
 #define HEXS_MERGE_ROWP 1
 #endif
+#ifndef HEXS_F2_2D
+#define HEXS_F2_2D 0  // 1 measured slower: heat2d5 1551 -> 1379 GUp/s, box2d9 1151 -> 946 (FADD2 holds
+                      // the FMA pipe 2 cycles, and the pair moves are IMADs on the same pipe)
+#endif
 #ifndef HEXS_MERGE_COLP
 #define HEXS_MERGE_COLP 0  // 1 measured slower: 1514 -> 1250 GUp/s star2d5
 #endif
@@ -85,6 +89,10 @@ struct Kernel {
   static constexpr int MINB = (sizeof(T) == 8 ? 8 : 12) / NW > 0 ? (sizeof(T) == 8 ? 8 : 12) / NW : 1;
   static constexpr int NIN = W0 + 4 * H + 5; // In rows per chunk (= In values per column)
   static constexpr int SW = C + 8;           // staged row width (elements), 16-B granular
+  // fp32 linear classes can sweep two columns per instruction (F2 pairs: FADD2 / FFMA2, see
+  // chunk_packed; the gradient's sqrt / div have no packed form) -- off by default, measured
+  // slower (HEXS_F2_2D above)
+  static constexpr bool kPacked = HEXS_F2_2D && std::is_same<T, float>::value && KIND != K_GRADIENT2D;
 
   struct Smem {
     uint64_t mbar[L];                 // one transaction barrier per level's In rows
@@ -176,6 +184,10 @@ struct Kernel {
   template <bool TMA, bool ROWP, bool COLP, bool TCUT>
   static __device__ __forceinline__ void chunk(const Fast2DArgs& g, Smem& sm, int64_t k, int64_t K,
                                                int64_t i0, const Coef<T>& cf) {
+    if constexpr (kPacked) {
+      chunk_packed<TMA, ROWP, COLP, TCUT>(g, sm, k, K, i0, cf);
+      return;
+    }
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
     const int64_t N0 = g.N0, N1 = g.N1;
     T in[Q][V + 2];  // input array of the current level: [row][halo0, halo1, own V]
@@ -272,11 +284,10 @@ struct Kernel {
           for (int r = 0; r < 3; ++r)
 #pragma unroll
             for (int c = 0; c < 3; ++c) x[r][c] = in[q - 1 + r][v + c];
-          const T val = apply<T, KIND>(x, cf);
-          if constexpr (ROWP || COLP) out[q][v] = (rowok && colok[v]) ? val : in[q][v + 1];
-          else out[q][v] = val;
+          out[q][v] = apply<T, KIND>(x, cf);
         }
-        // interleaved copy-out of the Out set (every row at the final level)
+        // interleaved copy-out of the Out set (every row at the final level); Dirichlet and
+        // out-of-domain cells are never stored
         if (is_out_row(a, q) || fin) {
           if (rowok) {
             T* rp = dbase + (int64_t)(q - 1) * N1;
@@ -285,14 +296,37 @@ struct Kernel {
               if (colok[v]) rp[v] = out[q][v];
           }
         }
-        // tail for the next warp / next super-chunk
-        if constexpr (a < L - 1) {
-          if (lane == 31) {
+      });
+      // Dirichlet cells keep their value: one branch per level instead of a select per
+      // element -- only the edge hexagons' levels that reach row 0 / N0-1 (CTA-uniform) and
+      // the threads holding a column outside [1, N1-2] enter it; the repaired values are the
+      // ones the next level and the tail see (out-of-domain cells feed only repaired cells)
+      if constexpr (ROWP || COLP) {
+        const bool rfix = ROWP && (i0 + (qlo - 1) < 1 || i0 + (qhi - 1) > N0 - 2);
+        bool cfix = false;
+#pragma unroll
+        for (int v = 0; v < V; ++v) cfix |= !colok[v];
+        if (rfix || cfix) {
+#pragma unroll
+          for (int q = qlo; q <= qhi; ++q) {
+            const int64_t row = i0 + (q - 1);
+            const bool rowok = !ROWP || (row >= 1 && row <= N0 - 2);
+#pragma unroll
+            for (int v = 0; v < V; ++v)
+              if (!(rowok && colok[v])) out[q][v] = in[q][v + 1];
+          }
+        }
+      }
+      // tail for the next warp / next super-chunk (one branch for all rows)
+      if constexpr (a < L - 1) {
+        if (lane == 31) {
+#pragma unroll
+          for (int q = qlo; q <= qhi; ++q) {
             sm.tail[k & 1][a][warp][q][0] = out[q][V - 2];
             sm.tail[k & 1][a][warp][q][1] = out[q][V - 1];
           }
         }
-      });
+      }
       __syncthreads();
       // ---- refill: the consumed slots of level a take chunk k+1's In rows ----
       if constexpr (TMA && n_in(a) > 0) {
@@ -306,6 +340,162 @@ struct Kernel {
       for (int q = qlo; q <= qhi; ++q)
 #pragma unroll
         for (int v = 0; v < V; ++v) in[q][v + 2] = out[q][v];
+    });
+  }
+
+  // The same super-chunk with the level held as F2 pairs (fp32 linear classes).  With in[0..5]
+  // the scalar path's input row (2 halo columns + the thread's 4), a row is held as
+  //   P[q][0] = (in0, in2), P[q][1] = (in1, in3), P[q][2] = (in2, in4), P[q][3] = (in3, in5)
+  // so the 3x3 operand window of outputs v and v+2 (p = v = 0, 1) is the pairs P[q-1..q+1]
+  // [p .. p+2] with no data movement, and the two output pairs (out0, out2), (out1, out3)
+  // ARE the next level's P[q][2], P[q][3]; P[q][0], P[q][1] take the left lane's out2 /
+  // out3 by shuffle plus one move each.  Every point is the scalar expression (stencil_ops,
+  // instantiated on F2), so results are bit-identical to the scalar sweep.
+  template <bool TMA, bool ROWP, bool COLP, bool TCUT>
+  static __device__ __forceinline__ void chunk_packed(const Fast2DArgs& g, Smem& sm, int64_t k, int64_t K,
+                                                      int64_t i0, const Coef<T>& cf) {
+    static_assert(V == 4, "packed sweep: fp32 quads");
+    const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
+    const int64_t N0 = g.N0, N1 = g.N1;
+    const Coef<F2> cf2{f2_pack((float)cf.k0, (float)cf.k0), f2_pack((float)cf.k1, (float)cf.k1)};
+    F2 P[Q][4];
+    auto set_row = [&](F2 (&r)[4], const T (&x)[V + 2]) {
+      r[0] = f2_pack(x[0], x[2]);
+      r[1] = f2_pack(x[1], x[3]);
+      r[2] = f2_pack(x[2], x[4]);
+      r[3] = f2_pack(x[3], x[5]);
+    };
+#pragma unroll
+    for (int q = 0; q < Q; ++q)
+#pragma unroll
+      for (int v = 0; v < 4; ++v) P[q][v] = f2_pack(0.f, 0.f);
+
+    static_for<0, L>([&](auto a_c) {
+      constexpr int a = decltype(a_c)::value;
+      if constexpr (TCUT) {
+        if (a < g.a_lo || a > g.a_hi) return;
+      }
+      const int64_t tau = g.tau0 + a;
+      const T* src = static_cast<const T*>(g.buf[tau & 1]);
+      T* dst = static_cast<T*>(g.buf[(tau + 1) & 1]);
+      const int colbase = (int)k * C - a + tid * V;
+      const bool first = TCUT ? (a == g.a_lo) : (a == 0);
+      if constexpr (TMA) {
+        static_assert(!TCUT, "TMA staging runs full-time tiles only");
+        if constexpr (n_in(a) > 0) mbar_wait_parity(&sm.mbar[a], (uint32_t)(k & 1));
+      }
+      const int pw = warp == 0 ? NW - 1 : warp - 1;
+      const int pk = warp == 0 ? (int)((k - 1) & 1) : (int)(k & 1);
+      auto halo = [&](auto q_c) {
+        constexpr int q = decltype(q_c)::value;
+        if constexpr (TMA && is_in_row(a, q)) {
+          constexpr int M = win_shift(a) - a - 1;
+          constexpr int NB = (M + V + 2 + VB - 1) / VB;
+          const T* rowp = &sm.inrows[in_slot(a, q)][tid * V];
+          T blk[NB * VB];
+#pragma unroll
+          for (int i = 0; i < NB; ++i) {
+            const float4 v4 = reinterpret_cast<const float4*>(rowp)[i];
+            blk[4 * i] = v4.x; blk[4 * i + 1] = v4.y; blk[4 * i + 2] = v4.z; blk[4 * i + 3] = v4.w;
+          }
+          T x[V + 2];
+#pragma unroll
+          for (int i = 0; i < V + 2; ++i) x[i] = blk[M + i];
+          set_row(P[q], x);
+        } else if constexpr (!TMA && is_input_row(a, q)) {
+          if (first || is_in_row(a, q)) {
+            int64_t row = i0 + (q - 1);
+            row = row < 0 ? 0 : (row >= N0 ? N0 - 1 : row);
+            T x[V + 2];
+            load_direct(src, N1, row, colbase - 1, x);
+            set_row(P[q], x);
+          }
+        }
+        if constexpr (is_input_row(a, q) && !is_in_row(a, q) && a > 0) {
+          if (!first) {
+            float c0, c2, c1, c3;
+            f2_unpack(P[q][2], c0, c2);  // own out0, out2 of level a-1
+            f2_unpack(P[q][3], c1, c3);  // own out1, out3
+            T h0 = __shfl_up_sync(0xffffffffu, c2, 1);
+            T h1 = __shfl_up_sync(0xffffffffu, c3, 1);
+            if (lane == 0) {
+              h0 = sm.tail[pk][a - 1][pw][q][0];
+              h1 = sm.tail[pk][a - 1][pw][q][1];
+            }
+            P[q][0] = f2_pack(h0, c0);
+            P[q][1] = f2_pack(h1, c1);
+          }
+        }
+      };
+      constexpr int qlo = lo_row(H, W0, a) + 1, qhi = hi_row(H, W0, a) + 1;
+      halo(std::integral_constant<int, qlo - 1>{});
+      halo(std::integral_constant<int, qlo>{});
+      F2 O[Q][2];
+      bool colok[V];
+#pragma unroll
+      for (int v = 0; v < V; ++v) {
+        const int c = colbase + v;
+        colok[v] = !COLP || (c >= 1 && c <= (int)N1 - 2);
+      }
+      const bool fin = TCUT && (a == g.a_final);
+      T* dbase = dst + i0 * N1 + colbase;
+      static_for<qlo, qhi + 1>([&](auto q_c) {
+        constexpr int q = decltype(q_c)::value;
+        halo(std::integral_constant<int, q + 1>{});
+        const int64_t row = i0 + (q - 1);
+        const bool rowok = !ROWP || (row >= 1 && row <= N0 - 2);
+        static_for<0, 2>([&](auto p_c) {
+          constexpr int p = decltype(p_c)::value;
+          F2 x[3][3];
+#pragma unroll
+          for (int r = 0; r < 3; ++r)
+#pragma unroll
+            for (int c = 0; c < 3; ++c) x[r][c] = P[q - 1 + r][p + c];
+          F2 val = apply<F2, KIND>(x, cf2);
+          if constexpr (ROWP || COLP) {
+            // keep (Dirichlet) old values: outputs p, p+2 hold in[p+1], in[p+3] = P[q][p+1]
+            float v0, v2, o0, o2;
+            f2_unpack(val, v0, v2);
+            f2_unpack(P[q][p + 1], o0, o2);
+            v0 = (rowok && colok[p]) ? v0 : o0;
+            v2 = (rowok && colok[p + 2]) ? v2 : o2;
+            val = f2_pack(v0, v2);
+          }
+          O[q][p] = val;
+        });
+        if (is_out_row(a, q) || fin) {
+          if (rowok) {
+            float o[4];
+            f2_unpack(O[q][0], o[0], o[2]);
+            f2_unpack(O[q][1], o[1], o[3]);
+            T* rp = dbase + (int64_t)(q - 1) * N1;
+#pragma unroll
+            for (int v = 0; v < V; ++v)
+              if (colok[v]) rp[v] = o[v];
+          }
+        }
+        if constexpr (a < L - 1) {
+          if (lane == 31) {
+            float o0, o2, o1, o3;
+            f2_unpack(O[q][0], o0, o2);
+            f2_unpack(O[q][1], o1, o3);
+            sm.tail[k & 1][a][warp][q][0] = o2;
+            sm.tail[k & 1][a][warp][q][1] = o3;
+          }
+        }
+      });
+      __syncthreads();
+      if constexpr (TMA && n_in(a) > 0) {
+        if (tid == 0 && k + 1 < K) {
+          fence_proxy_async_smem();
+          issue_level(g, sm, k + 1, a, i0);
+        }
+      }
+#pragma unroll
+      for (int q = qlo; q <= qhi; ++q) {
+        P[q][2] = O[q][0];
+        P[q][3] = O[q][1];
+      }
     });
   }
 

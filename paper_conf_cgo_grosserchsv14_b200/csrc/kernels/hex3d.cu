@@ -134,6 +134,15 @@ __device__ __forceinline__ void tma_3d(void* dst, const CUtensorMap* map, int x,
       : "memory");
 }
 
+// fp32 star sweeps evaluate two x columns per instruction (F2: FADD2 / FFMA2,
+// stencil_ops.cuh); gradient (sqrt / div) and 27-point (9 shifted lines: more moves and
+// spills than FP instructions saved, SASS-checked) stay scalar.  HEXS_F2=0: scalar.
+#ifndef HEXS_F2
+#define HEXS_F2 0  // 1 measured neutral on heat-3D 512^3 (552 vs 552 GUp/s): the sweep is not FP-issue bound
+#endif
+template <typename T, int KIND>
+constexpr bool kPacked3 = HEXS_F2 && std::is_same<T, float>::value && KIND == K_STAR3D7;
+
 template <typename T, int KIND>
 __device__ __forceinline__ T apply(const T (&x)[3][3][3], const Coef<T>& k) {
   // x[dz][dy][dx], offsets -1..1
@@ -469,6 +478,8 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
   // ================= compute warps =================
   uint32_t ph = 0u;  // parity bit per buffer
   const Coef<T> cf{(T)g.k0, (T)g.k1};
+  [[maybe_unused]] Coef<F2> cf2;
+  if constexpr (kPacked3<T, KIND>) cf2 = Coef<F2>{f2_pack((float)g.k0, (float)g.k0), f2_pack((float)g.k1, (float)g.k1)};
   const int lane = tid & 31;
   int slot = 0, ctile = 0;
   while (true) {
@@ -563,6 +574,26 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
           // one output row i from the windows of rows i-1, i, i+1 (registers)
           auto step = [&](int i, const Win<T>& wm, const Win<T>& wc, const Win<T>& wp) {
             T out[4];
+            if constexpr (kPacked3<T, KIND>) {
+              // x columns (2p, 2p+1) as one F2 pair: the centre-column operands are the
+              // LDS.128 quad's own register pairs, the x-shifted ones one move each
+#pragma unroll
+              for (int p = 0; p < 2; ++p) {
+                F2 x[3][3][3];
+#pragma unroll
+                for (int dy = 0; dy < 3; ++dy)
+#pragma unroll
+                  for (int dx = 0; dx < 3; ++dx) {
+                    x[0][dy][dx] = f2_pack(wm.v[dy][2 * p + dx], wm.v[dy][2 * p + dx + 1]);
+                    x[1][dy][dx] = f2_pack(wc.v[dy][2 * p + dx], wc.v[dy][2 * p + dx + 1]);
+                    x[2][dy][dx] = f2_pack(wp.v[dy][2 * p + dx], wp.v[dy][2 * p + dx + 1]);
+                  }
+                float o0, o1;
+                f2_unpack(apply<F2, KIND>(x, cf2), o0, o1);
+                out[2 * p] = o0;
+                out[2 * p + 1] = o1;
+              }
+            } else {
 #pragma unroll
             for (int j = 0; j < 4; ++j) {
               T x[3][3][3];
@@ -575,6 +606,7 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
                   x[2][dy][dx] = wp.v[dy][j + dx];
                 }
               out[j] = apply<T, KIND>(x, cf);
+            }
             }
             out[0] = xl ? wc.v[1][1] : out[0];
             out[3] = xr ? wc.v[1][4] : out[3];

@@ -22,6 +22,37 @@ enum Kind : int {
 
 template <typename T> struct Coef { T k0, k1; };
 
+// Blackwell packed FP32 (sm_100a FADD2 / FMUL2): a pair of fp32 values in one 64-bit
+// register pair; each operator is two IEEE round-to-nearest fp32 operations in ONE
+// instruction, element-wise bit-identical to the scalar ones (no FTZ, no contraction).
+// The per-class expressions below, instantiated on F2, evaluate two points with the same
+// association order -- half the FP32 instructions of the scalar sweep.
+struct F2 { uint64_t v; };
+__device__ __forceinline__ F2 f2_pack(float a, float b) {
+  F2 r;
+  asm("mov.b64 %0, {%1, %2};" : "=l"(r.v) : "f"(a), "f"(b));
+  return r;
+}
+__device__ __forceinline__ void f2_unpack(F2 p, float& a, float& b) {
+  asm("mov.b64 {%0, %1}, %2;" : "=f"(a), "=f"(b) : "l"(p.v));
+}
+__device__ __forceinline__ F2 operator+(F2 a, F2 b) {
+  F2 d;
+  asm("add.rn.f32x2 %0, %1, %2;" : "=l"(d.v) : "l"(a.v), "l"(b.v));
+  return d;
+}
+// ptxas contracts mul.rn.f32x2 feeding add.rn.f32x2 into FFMA2 even under --fmad=false
+// (probed: tools/probe_f32x2/contract.cu), which would round k0*c and the sum once instead
+// of twice.  So the product is an FFMA2 whose addend is -0.0 read from constant memory:
+// a*b + (-0) == a*b bit for bit (RN, no FTZ; +0 + -0 = +0), and an FMA result cannot be
+// contracted again.
+static __constant__ uint64_t kF2NegZero = 0x8000000080000000ull;
+__device__ __forceinline__ F2 operator*(F2 a, F2 b) {
+  F2 d;
+  asm("fma.rn.f32x2 %0, %1, %2, %3;" : "=l"(d.v) : "l"(a.v), "l"(b.v), "l"(kF2NegZero));
+  return d;
+}
+
 template <typename T> __device__ __forceinline__ T dev_sqrt(T x);
 template <> __device__ __forceinline__ float dev_sqrt<float>(float x) { return __fsqrt_rn(x); }
 template <> __device__ __forceinline__ double dev_sqrt<double>(double x) { return __dsqrt_rn(x); }
