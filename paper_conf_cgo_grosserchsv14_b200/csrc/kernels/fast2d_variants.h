@@ -29,5 +29,7 @@
   X(22, 0, float, K_STAR2D5, 2, 7, 4)            \
   X(23, 0, float, K_STAR2D5, 2, 9, 4)            \
   X(24, 0, float, K_BOX2D9, 2, 9, 4)             \
-  X(25, 0, float, K_STAR2D5, 3, 9, 4)
-#define HEXS_FAST2D_COUNT 26
+  X(25, 0, float, K_STAR2D5, 3, 9, 4)          \
+  X(26, 0, float, K_STAR2D5, 2, 8, 4)          \
+  X(27, 0, float, K_STAR2D5, 2, 6, 4)
+#define HEXS_FAST2D_COUNT 28

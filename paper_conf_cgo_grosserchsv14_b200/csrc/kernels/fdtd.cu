@@ -24,6 +24,7 @@
 //     its C final columns of every row the hexagon modifies are written back with coalesced
 //     stores -- the interleaved copy-out of Sec. 4.2.1.
 #include <cstdint>
+#include <type_traits>
 
 #include "../stencil_ops.cuh"
 #include "devcache.h"
@@ -33,6 +34,12 @@ namespace hexs {
 namespace fdtd {
 
 constexpr int C = 64;        // columns per chunk (= ring block)
+#ifndef HEXS_FDTD_PAIR
+#define HEXS_FDTD_PAIR 1  // ey and ex of a time step in one barrier interval (unrolled kernel)
+#endif
+#ifndef HEXS_FDTD_UNROLL
+#define HEXS_FDTD_UNROLL 1  // 0: the run-time-row kernel for every tile
+#endif
 #ifndef HEXS_FDTD_RING
 #define HEXS_FDTD_RING 4  // 3 (3 CTAs/SM, one-chunk prefetch) measured 226 -> 192 GUp/s
 #endif
@@ -67,8 +74,37 @@ __device__ __forceinline__ void cp_async_wait() {
 __device__ __forceinline__ int64_t max64(int64_t a, int64_t b) { return a > b ? a : b; }
 __device__ __forceinline__ int64_t min64(int64_t a, int64_t b) { return a < b ? a : b; }
 
+// Compile-time hexagon of the FDTD schedule (delta0 = 1, delta1 = 1/2, reading R15): the row
+// range of level a, SURVEY 8(a)'s closed form of eqs. (6)-(13) with F0 = h, F1 = floor(h/2),
+// e1 = 1/2, e0 = 0.  The host checks it against the plan's rows before choosing the unrolled
+// kernel (fdtd_unrolled_ok).
+template <int H, int W0> struct FHex {
+  static constexpr int L = 2 * H + 2, F0 = H, F1 = H / 2, W = 2 * W0 + 2 + F0 + F1;
+  __host__ __device__ static constexpr int cdiv2(int x) { return x >= 0 ? (x + 1) / 2 : -((-x) / 2); }  // ceil(x / 2)
+  __host__ __device__ static constexpr int fdiv2(int x) { return x >= 0 ? x / 2 : -((-x + 1) / 2); }   // floor(x / 2)
+  __host__ __device__ static constexpr int lo(int a) {
+    const int l1 = a - (2 * H + 1) + F0, l2 = cdiv2(H - 1 - a);
+    return l1 > l2 ? l1 : l2;
+  }
+  __host__ __device__ static constexpr int hi(int a) {
+    const int h1 = fdiv2(2 * H + 1 - a) + F0 + W0, h2 = a - H + F0 + F1 + W0;
+    return h1 < h2 ? h1 : h2;
+  }
+};
+template <int A, int N, class F>
+__device__ __forceinline__ void static_for(F&& f) {
+  if constexpr (A < N) {
+    f(std::integral_constant<int, A>{});
+    static_for<A + 1, N>(f);
+  }
+}
+
 // fields: 0 = ex, 1 = ey, 2 = hz (the order of FdtdArgs::f); statement k: 0 ey, 1 ex, 2 hz
-template <typename T>
+// UH > 0: the levels and their row ranges are compile-time (hexagon (UH, UW0), launches start
+// at tau0 = 0 mod 3): every level is unrolled with its rows spread over the RP row parts as
+// immediate shared-memory offsets -- no per-level table reads, no run-time trip counts.
+// UH = 0: any (h, w0), rows from the kernel arguments.
+template <typename T, int UH, int UW0>
 __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ FdtdArgs g) {
   extern __shared__ __align__(16) unsigned char smem_raw[];
   T* ring = reinterpret_cast<T*>(smem_raw);
@@ -145,6 +181,66 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
     stage(k + NB - 1);     // a later chunk's new block (ring slot of block k-1, written back)
     cp_async_wait<1>();    // every block but the newest has landed
     __syncthreads();
+    if constexpr (UH > 0) {
+      using HX = FHex<UH, UW0>;
+      // all rows of the three fields hold (b + 1) * RC + ring column offsets from a per-level base
+      static_for<0, HX::L>([&](auto a_c) {
+        constexpr int a = decltype(a_c)::value;
+        constexpr int st = a % 3, LO = HX::lo(a), HI = HX::hi(a);
+        constexpr int M = (HI - LO + RP) / RP;  // row slots per thread (the last one predicated)
+        if (a < g.a_lo || a > g.a_hi) return;   // time-cut launches (CTA-uniform)
+        const int blo = max(LO, st == 0 ? (int)(1 - i0) : (int)(-i0));
+        const int bhi = min(HI, st == 2 ? (int)(N0 - 2 - i0) : (int)(N0 - 1 - i0));
+        const int j = k * C - a + col;
+        const int cj = ring_col(j);
+        const bool jok = j >= (st == 1 ? 1 : 0) && j <= (st == 2 ? (int)N1 - 2 : (int)N1 - 1);
+        // rows b = LO + rpar + RP m; slot m valid iff blo <= b <= bhi
+        const int base = (LO + 1 + rpar) * RC + cj;
+        if (jok) {
+          if constexpr (st == 0) {  // ey[i][j] -= ce * (hz[i][j] - hz[i-1][j])
+#pragma unroll
+            for (int m = 0; m < M; ++m) {
+              const int b = LO + rpar + RP * m;
+              if (b >= blo && b <= bhi) {
+                T* pe = ring + R * RC + base + RP * m * RC;
+                const T* ph = ring + 2 * R * RC + base + RP * m * RC;
+                *pe = fdtd_ey<T>(*pe, ph[0], ph[-RC], cf);
+              }
+            }
+          } else if constexpr (st == 1) {  // ex[i][j] -= ce * (hz[i][j] - hz[i][j-1])
+            const int dm = ring_col(j - 1) - cj;
+#pragma unroll
+            for (int m = 0; m < M; ++m) {
+              const int b = LO + rpar + RP * m;
+              if (b >= blo && b <= bhi) {
+                T* px = ring + base + RP * m * RC;
+                const T* ph = ring + 2 * R * RC + base + RP * m * RC;
+                *px = fdtd_ex<T>(*px, ph[0], ph[dm], cf);
+              }
+            }
+          } else {  // hz[i][j] -= ch * (((ex[i][j+1] - ex[i][j]) + ey[i+1][j]) - ey[i][j])
+            const int dp = ring_col(j + 1) - cj;
+#pragma unroll
+            for (int m = 0; m < M; ++m) {
+              const int b = LO + rpar + RP * m;
+              if (b >= blo && b <= bhi) {
+                T* ph = ring + 2 * R * RC + base + RP * m * RC;
+                const T* px = ring + base + RP * m * RC;
+                const T* pe = ring + R * RC + base + RP * m * RC;
+                *ph = fdtd_hz<T>(*ph, px[dp], px[0], pe[RC], pe[0], cf);
+              }
+            }
+          }
+        }
+        // ey (tau = 3t) and ex (3t + 1) read only hz of step t-1 and write different fields:
+        // one barrier interval holds both (2 barriers per time step instead of 3)
+        if constexpr (st != 0 || !HEXS_FDTD_PAIR) {
+          __syncthreads();
+        } else {
+          if (a == g.a_hi) __syncthreads();  // a launch's last level: before the write-back
+        }
+      });
+    } else {
     int st = (int)((g.tau0 + g.a_lo) % 3);
     for (int l = 0; l < nlev; ++l, st = st == 2 ? 0 : st + 1) {
       // level parameters from the kernel arguments (constant bank), clipped to the grid and the
@@ -188,6 +284,7 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
       }
       __syncthreads();
     }
+    }
     // write back the columns no later chunk touches: [kC - a_hi, (k+1)C - a_hi), or all
     // remaining columns after the last chunk
     const int wlo = max(0, k * C - g.a_hi);
@@ -209,6 +306,17 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
   cp_async_wait<0>();
 }
 
+// the compiled unrolled hexagon (the default FDTD tile, plan.cpp) applies when the plan's
+// rows are exactly its rows and the launch starts a time step (statement order ey, ex, hz)
+constexpr int kUH = 11, kUW0 = 5;
+bool unrolled_ok(const FdtdArgs& a) {
+  using HX = FHex<kUH, kUW0>;
+  if (a.W != HX::W || a.tau0 % 3 != 0) return false;
+  for (int q = 0; q < HX::L; ++q)
+    if (a.lo[q] != HX::lo(q) || a.hi[q] != HX::hi(q)) return false;
+  return true;
+}
+
 template <typename T>
 cudaError_t launch_t(const FdtdArgs& a, int grid, cudaStream_t s) {
   // per device: opt in once to the largest ring any plan can ask for (fdtd_variant caps it)
@@ -218,10 +326,16 @@ cudaError_t launch_t(const FdtdArgs& a, int grid, cudaStream_t s) {
   int done = 0;
   cudaError_t e = attr.get(&done, [](int, int* v) {
     *v = 1;
-    return cudaFuncSetAttribute(fdtd_kernel<T>, cudaFuncAttributeMaxDynamicSharedMemorySize, 200 * 1024);
+    cudaError_t r = cudaFuncSetAttribute(fdtd_kernel<T, 0, 0>, cudaFuncAttributeMaxDynamicSharedMemorySize, 200 * 1024);
+    if (r == cudaSuccess)
+      r = cudaFuncSetAttribute(fdtd_kernel<T, kUH, kUW0>, cudaFuncAttributeMaxDynamicSharedMemorySize, 200 * 1024);
+    return r;
   });
   if (e != cudaSuccess) return e;
-  fdtd_kernel<T><<<grid, NT, smem, s>>>(a);
+  if (HEXS_FDTD_UNROLL && unrolled_ok(a))
+    fdtd_kernel<T, kUH, kUW0><<<grid, NT, smem, s>>>(a);
+  else
+    fdtd_kernel<T, 0, 0><<<grid, NT, smem, s>>>(a);
   return cudaGetLastError();
 }
 

@@ -12,7 +12,8 @@
 //           (constraint-based unrolling), so their code grows with P; once a
 //           body outgrows the instruction cache the SM starves for instructions (ncu stall
 //           "no_instruction") -- factor min(1, C / S)^3, S = P * (4 * flops + 6|10) * 16 bytes,
-//           C = 44 000 B (2D register-wavefront kernel) / 58 000 B (3D tile-wavefront kernel),
+//           C = 39 000 B (2D register-wavefront kernel; 44 000 before the round-2 select-free
+//           body made (2,7) beat (3,7) for star2d5) / 58 000 B (3D tile-wavefront kernel),
 //           fitted to the sweeps;
 //           (2) CTA count: a launch of n hexagon CTAs on `slots` resident slots runs
 //           ceil(n / slots) waves -- factor n / (waves * slots) (grid quantisation).
@@ -100,7 +101,7 @@ bool tile_eval(const Desc& d, int hd, const Rat& d0, const Rat& d1, int h, int w
   // per-row data movement (shuffles, shared loads, stores): 6 (2D) / 10 (3D) instructions of 16 B
   const double per_row = family == FAMILY_FAST2D ? 4.0 * flops_of(d.kind) + 6.0 : 4.0 * flops_of(d.kind) + 10.0;
   e.body_bytes = family == FAMILY_GENERIC ? 0.0 : (double)P * per_row * 16.0;
-  const double cap = family == FAMILY_FAST2D ? 44000.0 : 58000.0;
+  const double cap = family == FAMILY_FAST2D ? 39000.0 : 58000.0;
   e.code_eff = family == FAMILY_GENERIC ? 1.0 : std::pow(std::min(1.0, cap / e.body_bytes), 3.0);
   // CTA count: one CTA per hexagon of a launch (2D fast and generic kernels: 3 resident per
   // SM); the 3D kernels are persistent over (hexagon, classical tile) items

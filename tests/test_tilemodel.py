@@ -17,8 +17,9 @@ def _eval(st, h, w0, family, hex_dim=0):
     return e
 
 
-# best (h, w0) measured on B200 among each class's compiled variants (profiles/round1/tile_sweep_*)
-MEASURED_BEST = [("star2d5", (8192, 8192), 1, (3, 7)), ("box2d9", (8192, 8192), 1, (2, 7)),
+# best (h, w0) measured on B200 among each class's compiled variants (profiles/round1/tile_sweep_*,
+# round 2: profiles/round2/tile_sweep_2d.txt -- star2d5 moved to (2, 7) with the select-free body)
+MEASURED_BEST = [("star2d5", (8192, 8192), 1, (2, 7)), ("box2d9", (8192, 8192), 1, (2, 7)),
                  ("gradient2d", (8192, 8192), 1, (1, 1)), ("star3d7", (512, 512, 512), 2, (3, 7))]
 
 
