@@ -57,7 +57,9 @@ constexpr int NT = RP * C;
 
 template <typename T>
 size_t smem_bytes(int W) {
-  return (size_t)3 * (W + 2) * RC * sizeof(T);
+  // three fields' ring rows, plus (unrolled kernel) RP + 2 padding rows that the row slots past a
+  // level's last row may read, plus one trash word per lane that their stores go to
+  return ((size_t)3 * (W + 2) * RC + (size_t)(RP + 2) * RC + 32) * sizeof(T);
 }
 
 __device__ __forceinline__ void cp_async16(void* dst, const void* src, bool valid) {
@@ -189,47 +191,57 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
         constexpr int st = a % 3, LO = HX::lo(a), HI = HX::hi(a);
         constexpr int M = (HI - LO + RP) / RP;  // row slots per thread (the last one predicated)
         if (a < g.a_lo || a > g.a_hi) return;   // time-cut launches (CTA-uniform)
-        const int blo = max(LO, st == 0 ? (int)(1 - i0) : (int)(-i0));
-        const int bhi = min(HI, st == 2 ? (int)(N0 - 2 - i0) : (int)(N0 - 1 - i0));
+        // Which slots store: cells outside the grid may compute anything -- they are never
+        // written back, and no in-grid cell reads one (ey[i] reads hz[i-1] for i >= 1, ex[j]
+        // hz[j-1] for j >= 1, hz[i][j] ex[j+1] / ey[i+1] inside the grid; staging zero-fills
+        // them) -- so only the in-grid cells a statement never updates (ey row 0, ex column 0,
+        // hz row N0-1 and column N1-1, the oracle's loop bounds) and the row slots past the
+        // level's last row are masked: one compare per slot, no table reads, no branches.
         const int j = k * C - a + col;
-        const int cj = ring_col(j);
-        const bool jok = j >= (st == 1 ? 1 : 0) && j <= (st == 2 ? (int)N1 - 2 : (int)N1 - 1);
-        // rows b = LO + rpar + RP m; slot m valid iff blo <= b <= bhi
-        const int base = (LO + 1 + rpar) * RC + cj;
-        if (jok) {
-          if constexpr (st == 0) {  // ey[i][j] -= ce * (hz[i][j] - hz[i-1][j])
+        const int cj = (int)((unsigned)(j + C) % (unsigned)RC);
+        bool lvok = true;  // column / last-slot conditions of this level
+        if constexpr (st == 1) lvok = j != 0;
+        if constexpr (st == 2) lvok = j != (int)N1 - 1;
+        constexpr int RR = HX::W + 2;  // ring rows per field (compile-time: immediate offsets)
+        T* const fb = ring + (LO + 1 + rpar) * RC + cj;  // field 0 (ex), row LO + rpar
+        T* const trash = ring + (3 * RR + RP + 2) * RC + (tid & 31);
+        constexpr int LASTLIM = HI - LO - RP * (M - 1);  // the last slot exists for rpar <= LASTLIM
+        const bool lastok = rpar <= LASTLIM;
+        auto slot_ok = [&](int m, int b) {
+          bool ok = lvok && (m < M - 1 || lastok);
+          if (st == 0) ok = ok && (b + (int)i0 != 0);
+          if (st == 2) ok = ok && (b + (int)i0 != (int)N0 - 1);
+          return ok;
+        };
+        if constexpr (st == 0) {  // ey[i][j] -= ce * (hz[i][j] - hz[i-1][j])
 #pragma unroll
-            for (int m = 0; m < M; ++m) {
-              const int b = LO + rpar + RP * m;
-              if (b >= blo && b <= bhi) {
-                T* pe = ring + R * RC + base + RP * m * RC;
-                const T* ph = ring + 2 * R * RC + base + RP * m * RC;
-                *pe = fdtd_ey<T>(*pe, ph[0], ph[-RC], cf);
-              }
-            }
-          } else if constexpr (st == 1) {  // ex[i][j] -= ce * (hz[i][j] - hz[i][j-1])
-            const int dm = ring_col(j - 1) - cj;
+          for (int m = 0; m < M; ++m) {
+            const int b = LO + rpar + RP * m;
+            T* pe = fb + (RR + RP * m) * RC;
+            const T* ph = fb + (2 * RR + RP * m) * RC;
+            const T v = fdtd_ey<T>(*pe, ph[0], ph[-RC], cf);
+            *(slot_ok(m, b) ? pe : trash) = v;
+          }
+        } else if constexpr (st == 1) {  // ex[i][j] -= ce * (hz[i][j] - hz[i][j-1])
+          const int dm = cj == 0 ? RC - 1 : -1;  // column j-1 in the ring
 #pragma unroll
-            for (int m = 0; m < M; ++m) {
-              const int b = LO + rpar + RP * m;
-              if (b >= blo && b <= bhi) {
-                T* px = ring + base + RP * m * RC;
-                const T* ph = ring + 2 * R * RC + base + RP * m * RC;
-                *px = fdtd_ex<T>(*px, ph[0], ph[dm], cf);
-              }
-            }
-          } else {  // hz[i][j] -= ch * (((ex[i][j+1] - ex[i][j]) + ey[i+1][j]) - ey[i][j])
-            const int dp = ring_col(j + 1) - cj;
+          for (int m = 0; m < M; ++m) {
+            const int b = LO + rpar + RP * m;
+            T* px = fb + (RP * m) * RC;
+            const T* ph = fb + (2 * RR + RP * m) * RC;
+            const T v = fdtd_ex<T>(*px, ph[0], ph[dm], cf);
+            *(slot_ok(m, b) ? px : trash) = v;
+          }
+        } else {  // hz[i][j] -= ch * (((ex[i][j+1] - ex[i][j]) + ey[i+1][j]) - ey[i][j])
+          const int dp = cj == RC - 1 ? 1 - RC : 1;  // column j+1 in the ring
 #pragma unroll
-            for (int m = 0; m < M; ++m) {
-              const int b = LO + rpar + RP * m;
-              if (b >= blo && b <= bhi) {
-                T* ph = ring + 2 * R * RC + base + RP * m * RC;
-                const T* px = ring + base + RP * m * RC;
-                const T* pe = ring + R * RC + base + RP * m * RC;
-                *ph = fdtd_hz<T>(*ph, px[dp], px[0], pe[RC], pe[0], cf);
-              }
-            }
+          for (int m = 0; m < M; ++m) {
+            const int b = LO + rpar + RP * m;
+            T* ph = fb + (2 * RR + RP * m) * RC;
+            const T* px = fb + (RP * m) * RC;
+            const T* pe = fb + (RR + RP * m) * RC;
+            const T v = fdtd_hz<T>(*ph, px[dp], px[0], pe[RC], pe[0], cf);
+            *(slot_ok(m, b) ? ph : trash) = v;
           }
         }
         // ey (tau = 3t) and ex (3t + 1) read only hz of step t-1 and write different fields:
@@ -292,6 +304,33 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
     for (int j = k * C - g.a_hi + col; j <= whi; j += C) {
       if (j < wlo) continue;
       const int cj = ring_col(j);
+      if constexpr (UH > 0) {
+        // compile-time row slots over each field's modified rows (union of its levels' rows),
+        // masked by the launch's clipped range [mlo, mhi]
+        using HX = FHex<UH, UW0>;
+        static_for<0, 3>([&](auto f_c) {
+          constexpr int f = decltype(f_c)::value;  // 0 ex (statement 1), 1 ey (0), 2 hz (2)
+          constexpr int stf = f == 0 ? 1 : (f == 1 ? 0 : 2);
+          constexpr int FLO = [] {
+            int v = 1 << 20;
+            for (int a = stf; a < HX::L; a += 3) v = HX::lo(a) < v ? HX::lo(a) : v;
+            return v;
+          }();
+          constexpr int FHI = [] {
+            int v = -1;
+            for (int a = stf; a < HX::L; a += 3) v = HX::hi(a) > v ? HX::hi(a) : v;
+            return v;
+          }();
+          constexpr int MF = (FHI - FLO + RP) / RP;
+          const T* sp = (f == 0 ? rex : (f == 1 ? rey : rhz)) + cj + (FLO + rpar) * RC;
+          T* gp = F[f] + ((i0 + FLO + rpar) * N1 + j);
+#pragma unroll
+          for (int m = 0; m < MF; ++m) {
+            const int b = FLO + rpar + RP * m;
+            if (b >= mlo[f] && b <= mhi[f]) gp[(int64_t)RP * m * N1] = sp[RP * m * RC];
+          }
+        });
+      } else {
 #pragma unroll
       for (int f = 0; f < 3; ++f) {
         const int b0 = mlo[f] + rpar;
@@ -299,6 +338,7 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
         T* gp = F[f] + ((i0 + b0) * N1 + j);
         const int64_t gstep = RP * N1;
         for (int b = b0; b <= mhi[f]; b += RP, sp += RP * RC, gp += gstep) *gp = *sp;
+      }
       }
     }
     __syncthreads();  // the write-back reads ring slots the next stage() overwrites
