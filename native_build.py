@@ -62,6 +62,8 @@ def _deps_hash(paths):
 
 EXTRA3D = []  # extra flags of the 3D kernel objects (debug builds)
 EXTRAS3 = []  # extra flags of the streaming 3D kernel objects
+EXTRA_ALL = []  # extra flags of the CUDA objects matching EXTRA_ONLY (experiment builds: --variant)
+EXTRA_ONLY = [""]
 
 
 def _units():
@@ -83,6 +85,9 @@ def _units():
     for vid in _variant_ids("stream3d_variants.h", "HEXS_STREAM3D_VARIANTS"):
         units.append((os.path.join(KDIR, "stream3d.cu"), "nvcc", [f"-DHEXS_S3_VARIANT={vid}"] + EXTRAS3))
     out = []
+    if EXTRA_ALL:
+        units = [(src, tool, extra + EXTRA_ALL if tool == "nvcc" and EXTRA_ONLY[0] in src else extra)
+                 for src, tool, extra in units]
     for src, tool, extra in units:
         key = _deps_hash([src] + headers) + hashlib.sha1(" ".join(extra).encode()).hexdigest()[:8]
         tags = [e.split("=")[-1] for e in extra if "=" in e]
@@ -143,7 +148,17 @@ def main():
                     help="also build lib/libhexstencil_tm.so with the 3D kernel's cycle accounting")
     ap.add_argument("--s3trace", action="store_true",
                     help="also build lib/libhexstencil_s3t.so with the streaming 3D kernel's event trace")
+    ap.add_argument("--variant", default="",
+                    help="build lib/libhexstencil_<VARIANT>.so with the -D flags below instead (experiments; "
+                         "load it with HEXS_LIB)")
+    ap.add_argument("-D", action="append", default=[], help="macro for the CUDA objects of --variant")
+    ap.add_argument("--only", default="", help="apply the -D flags only to sources whose path contains this")
     args = ap.parse_args()
+    if args.variant:
+        EXTRA_ALL.extend("-D" + d for d in args.D)
+        EXTRA_ONLY[0] = args.only
+        print(build_library(args.j, args.v, lib=os.path.join(PKG, "lib", f"libhexstencil_{args.variant}.so")))
+        return
     print(build_library(args.j, args.v))
     if args.s3trace:
         EXTRAS3.append("-DHEXS_S3_TRACE")

@@ -117,6 +117,7 @@ struct Plan {
   int64_t tile_points = 0, tile_in = 0, tile_out = 0;
   bool wavefront = false;      // generic executor: classical tiles as a dependence wavefront
   size_t flag_off = 0, counter_off = 0, flag_bytes = 0;  // workspace layout (wavefront)
+  int64_t n_counters = 0;  // ticket counters; the completed-tile counters follow them
   // stream3d: per-launch progress counters + ticket (zeroed per run), carry scratch
   size_t s3_ctr_off = 0, s3_ctr_bytes = 0, s3_scratch_off = 0;
   int s3_nstr = 0;

@@ -304,33 +304,6 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
     for (int j = k * C - g.a_hi + col; j <= whi; j += C) {
       if (j < wlo) continue;
       const int cj = ring_col(j);
-      if constexpr (UH > 0) {
-        // compile-time row slots over each field's modified rows (union of its levels' rows),
-        // masked by the launch's clipped range [mlo, mhi]
-        using HX = FHex<UH, UW0>;
-        static_for<0, 3>([&](auto f_c) {
-          constexpr int f = decltype(f_c)::value;  // 0 ex (statement 1), 1 ey (0), 2 hz (2)
-          constexpr int stf = f == 0 ? 1 : (f == 1 ? 0 : 2);
-          constexpr int FLO = [] {
-            int v = 1 << 20;
-            for (int a = stf; a < HX::L; a += 3) v = HX::lo(a) < v ? HX::lo(a) : v;
-            return v;
-          }();
-          constexpr int FHI = [] {
-            int v = -1;
-            for (int a = stf; a < HX::L; a += 3) v = HX::hi(a) > v ? HX::hi(a) : v;
-            return v;
-          }();
-          constexpr int MF = (FHI - FLO + RP) / RP;
-          const T* sp = (f == 0 ? rex : (f == 1 ? rey : rhz)) + cj + (FLO + rpar) * RC;
-          T* gp = F[f] + ((i0 + FLO + rpar) * N1 + j);
-#pragma unroll
-          for (int m = 0; m < MF; ++m) {
-            const int b = FLO + rpar + RP * m;
-            if (b >= mlo[f] && b <= mhi[f]) gp[(int64_t)RP * m * N1] = sp[RP * m * RC];
-          }
-        });
-      } else {
 #pragma unroll
       for (int f = 0; f < 3; ++f) {
         const int b0 = mlo[f] + rpar;
@@ -338,7 +311,6 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
         T* gp = F[f] + ((i0 + b0) * N1 + j);
         const int64_t gstep = RP * N1;
         for (int b = b0; b <= mhi[f]; b += RP, sp += RP * RC, gp += gstep) *gp = *sp;
-      }
       }
     }
     __syncthreads();  // the write-back reads ring slots the next stage() overwrites

@@ -121,6 +121,11 @@ __device__ __forceinline__ int ld_acquire(const int* p) {
   asm volatile("ld.acquire.gpu.global.b32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
   return v;
 }
+__device__ __forceinline__ int ld_relaxed(const int* p) {
+  int v;
+  asm volatile("ld.relaxed.gpu.global.b32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
+  return v;
+}
 __device__ __forceinline__ void st_release(int* p, int v) {
   asm volatile("st.release.gpu.global.b32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
 }
@@ -321,6 +326,8 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
   const int sts_off = ly * NXP + 4 * q;                  // + row * MAIN in the output buffer
   const bool cthr = (ly >= LNY - 2) || (q >= NQ - 2);   // writes its successors' carries
 
+  // chained launches: the next launch may be scheduled as soon as every CTA of this one runs
+  if (g.pdl) asm volatile("griddepcontrol.launch_dependents;" ::: "memory");
   if (tid == 0) {
     mbar_init(&full[0], 1);
     mbar_init(&full[1], 1);
@@ -420,6 +427,64 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
     tma_3d(buf_of(b) + LY::EDGE_OFF, &mp.carry[par], xo - 4, yo - 1 - SC<T>, z0, &full[b]);
   };
 
+  // Chained mode: a tile reads, at every level a, z rows [i0 - 1, i0 + Q - 2], y lines
+  // [Y0 - a - 1, Y0 - a + NY] and x [X0 - 4a - 1, X0 - 4a + NX] of time tau0 + a.  A writer
+  // launch with base time tau0' computed that time at its level a' = a + D, D = tau0 - tau0' - 1,
+  // where its tile (S1', S2') covers y [S1' NY - a', S1' NY - a' + NY - 1] and x
+  // [S2' NX - 4a', S2' NX - 4a' + NX - 1]; intersecting gives a range of S1' / S2' that does not
+  // depend on a, and hexagon S0' covers rows [S0' W - row_off', S0' W - row_off' + Q - 3].
+  // Every such writer tile that exists is acquired (a superset of the true producers).
+  auto fdiv = [](int64_t x, int64_t y) { return x >= 0 ? x / y : -((-x + y - 1) / y); };
+  // (producer lane) launches seen complete need no more polls: their completed-tile counter
+  // reached their tile count once, and the fence after that observation is the acquire
+  bool prev_done[2] = {g.prev[0].flags == nullptr, g.prev[1].flags == nullptr};
+  auto wait_prev = [&](const long long* it) {
+    if (prev_done[0] && prev_done[1]) return;
+    bool fresh = false;
+    for (int k = 0; k < 2; ++k) {
+      const Fast3DPrev& pv = g.prev[k];
+      if (prev_done[k]) continue;
+      unsigned long long d;
+      asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(d) : "l"(pv.done) : "memory");
+      if (d == (unsigned long long)((pv.S0_hi - pv.S0_lo + 1) * pv.n1 * pv.n2)) prev_done[k] = fresh = true;
+    }
+    if (prev_done[0] && prev_done[1]) {
+      if (fresh) __threadfence();
+      return;
+    }
+    int64_t i0;
+    int X0, Y0;
+    tile_origin(it, i0, X0, Y0);
+    const int64_t S1r = Y0 / LNY, S2r = X0 / NX;
+    for (int k = 0; k < 2; ++k) {
+      const Fast3DPrev& pv = g.prev[k];
+      if (prev_done[k]) continue;
+      const int64_t D = g.tau0 - pv.tau0 - 1;
+      const int64_t zlo = i0 - 1, zhi = i0 + g.Q - 2;
+      int64_t s0a = -fdiv(-(zlo - (g.Q - 3) + pv.row_off), g.W), s0b = fdiv(zhi + pv.row_off, g.W);
+      int64_t s1a = -fdiv(-(S1r * LNY - LNY + D), LNY), s1b = fdiv(S1r * LNY + LNY + D, LNY);
+      int64_t s2a = -fdiv(-(S2r * NX - NX + SIGMA * D), NX), s2b = fdiv(S2r * NX + NX + SIGMA * D, NX);
+      s0a = s0a < pv.S0_lo ? pv.S0_lo : s0a;
+      s0b = s0b > pv.S0_hi ? pv.S0_hi : s0b;
+      s1a = s1a < pv.S1_lo ? pv.S1_lo : s1a;
+      s1b = s1b > pv.S1_lo + pv.n1 - 1 ? pv.S1_lo + pv.n1 - 1 : s1b;
+      s2a = s2a < pv.S2_lo ? pv.S2_lo : s2a;
+      s2b = s2b > pv.S2_lo + pv.n2 - 1 ? pv.S2_lo + pv.n2 - 1 : s2b;
+      // relaxed polls, all in flight at once (an acquire load per flag would serialise ~20 L2
+      // round trips per tile); one fence after the last flag is seen gives the acquire
+      bool all = false;
+      while (!all) {
+        all = true;
+        for (int64_t s0 = s0a; s0 <= s0b; ++s0)
+          for (int64_t s1 = s1a; s1 <= s1b; ++s1)
+            for (int64_t s2 = s2a; s2 <= s2b; ++s2)
+              all &= ld_relaxed(pv.flags + ((s0 - pv.S0_lo) * pv.n1 + (s1 - pv.S1_lo)) * pv.n2 + (s2 - pv.S2_lo)) != 0;
+        if (!all) __nanosleep(128);
+      }
+    }
+    __threadfence();  // acquire: the writers' stores (released with their flags) happen before our reads
+  };
+
   F3_TM_DECL
   if (tid >= NC) {
     // ================= producer warp (one lane): tiles, predecessor flags, TMA =================
@@ -447,15 +512,27 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
           F3_TM(0);
           fence_proxy_async_smem();
           if (a == a_lo) {
+            if (g.prev[0].flags) {  // chained: the previous launches' writers of this tile's inputs
+              F3_TR(3, ptile, a);
+              wait_prev(it);
+              fence_proxy_async_global();
+              F3_TR(4, ptile, a);
+            }
             issue_first(it, a);
           } else {
             if (a == a_lo + 1) {  // predecessors complete: their carries are in global memory
               F3_TR(3, ptile, a);
+              // both predecessors polled together (relaxed loads in flight at once), then one
+              // fence: the acquire of their carries
               const int* f = g.flags + base;
-              if (it[1] > 0)
-                while (ld_acquire(f + (it[1] - 1) * n2 + it[2]) == 0) __nanosleep(64);
-              if (it[2] > 0)
-                while (ld_acquire(f + it[1] * n2 + it[2] - 1) == 0) __nanosleep(64);
+              const int* fy = it[1] > 0 ? f + (it[1] - 1) * n2 + it[2] : nullptr;
+              const int* fx = it[2] > 0 ? f + it[1] * n2 + it[2] - 1 : nullptr;
+              while (true) {
+                const int vy = fy ? ld_relaxed(fy) : 1, vx = fx ? ld_relaxed(fx) : 1;
+                if (vy != 0 && vx != 0) break;
+                __nanosleep(64);
+              }
+              if (fy || fx) __threadfence();
               fence_proxy_async_global();
               F3_TR(4, ptile, a);
               F3_TM(2);
@@ -723,7 +800,11 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
     }
     named_barrier_sync(1, NC);  // every compute thread's stores of the tile are issued
     F3_TM(1);
-    if (tid == 0) st_release(my_flag, 1);
+    if (tid == 0) {
+      st_release(my_flag, 1);
+      // chained mode: count the launch's completed tiles (release: after the tile's stores)
+      if (g.done) asm volatile("red.release.gpu.global.add.u64 [%0], 1;" ::"l"(g.done) : "memory");
+    }
     if (tid == 0) F3_TR(8, ctile, 0);
     ++ctile;
     slot ^= 1;
@@ -785,6 +866,20 @@ cudaError_t launch_t(const Fast3DArgs& a, cudaStream_t s) {
   }
   const int64_t items = (a.S0_hi - a.S0_lo + 1) * a.n1 * a.n2;
   const int gsz = (int)(items < grid ? items : grid);
+  if (a.pdl) {
+    // chained launch: may start while the previous launch drains (its tiles wait on flags)
+    cudaLaunchConfig_t cfg = {};
+    cfg.gridDim = dim3((unsigned)gsz);
+    cfg.blockDim = dim3((unsigned)NT);
+    cfg.dynamicSmemBytes = smem;
+    cfg.stream = s;
+    cudaLaunchAttribute at[1];
+    at[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+    at[0].val.programmaticStreamSerializationAllowed = 1;
+    cfg.attrs = at;
+    cfg.numAttrs = 1;
+    return cudaLaunchKernelEx(&cfg, kern, a, m);
+  }
   kern<<<gsz, NT, smem, s>>>(a, m);
   return cudaGetLastError();
 }

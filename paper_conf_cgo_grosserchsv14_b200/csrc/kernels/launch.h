@@ -87,6 +87,12 @@ int fdtd_ctas_per_sm();  // resident CTAs per SM the FDTD kernel is built for
 // 3D fast kernel (kernels/hex3d.cu): persistent CTAs run the classical tiles of every
 // hexagon of the launch as a tile-granular dependence wavefront, all levels of a tile in
 // shared memory.
+// A launch whose tiles a 3D launch reads (chained mode): its tile flags and tile geometry.
+struct Fast3DPrev {
+  const int* flags;  // nullptr: none
+  const unsigned long long* done;  // its completed-tile counter (== its tile count: all complete)
+  int64_t tau0, S0_lo, S0_hi, row_off, S1_lo, n1, S2_lo, n2;
+};
 struct Fast3DArgs {
   void* buf[2];
   int64_t N0, N1, N2;
@@ -106,6 +112,12 @@ struct Fast3DArgs {
   int mir_y0[2];
   int mir_G;
   int mir_fence;  // 1: each thread that stored into a mirror fences at system scope before the tile's flag
+  // Chained launches (single GPU): the launch may start while the previous two are still running
+  // (programmatic dependent launch); before a tile's first fill its producer acquires the flags of
+  // every tile of prev[0] (launch - 1) and prev[1] (launch - 2) that wrote a value it reads.
+  Fast3DPrev prev[2];
+  unsigned long long* done;  // this launch's completed-tile counter (chained mode; else nullptr)
+  int pdl;  // 1: launched with programmatic stream serialization (and lets the next launch start early)
 };
 cudaError_t launch_fast3d(int variant, const Fast3DArgs& a, int grid, cudaStream_t s);
 constexpr int kFast3DNX = 32;            // classical tile width along x of the 3D fast kernel

@@ -399,7 +399,9 @@ stencil_status build_plan(const Desc& d, int64_t T_steps, const stencil_tile_t* 
     }
     p->flag_off = p->ws_bytes;
     p->counter_off = p->flag_off + ((size_t)n_items * sizeof(int) + 255) / 256 * 256;
-    p->flag_bytes = p->counter_off - p->flag_off + ((size_t)idx * 8 + 255) / 256 * 256;  // flags + counters
+    // flags + ticket counters + per-launch completed-tile counters (3D chained launches)
+    p->flag_bytes = p->counter_off - p->flag_off + ((size_t)idx * 16 + 255) / 256 * 256;
+    p->n_counters = idx;
     p->ws_bytes = p->flag_off + p->flag_bytes;
   }
   // streaming 3D kernel: per launch a progress counter per (hexagon, strip) CTA plus a ticket

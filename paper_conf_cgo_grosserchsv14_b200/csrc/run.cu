@@ -104,6 +104,11 @@ stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* 
   };
   cudaStream_t s = static_cast<cudaStream_t>(stream_);
   const size_t bytes = (size_t)d.points() * d.elem();
+  // HEXS_F3_CHAIN=0: 3D launches strictly one after the other (no cross-launch overlap)
+  static const bool f3_chain = [] {
+    const char* e = getenv("HEXS_F3_CHAIN");
+    return !(e && e[0] == '0');
+  }();
   int dev = -1;
   HEXS_CUDA(cudaGetDevice(&dev), "stencil_run: no CUDA device");
   HEXS_CUDA(cudaGetLastError(), "stencil_run: pending CUDA error");
@@ -291,6 +296,29 @@ stencil_status run_plan(Plan& p, const void* const* in, void* const* out, void* 
         a.mir_G = p.mir_G;
         a.mir_fence = p.mir_fence;
         a.counter = reinterpret_cast<unsigned long long*>(ws + p.counter_off) + l.counter_idx;
+        // chained launches (single GPU): launch k may start while k-1 drains; its tiles acquire
+        // the flags of the tiles of k-1 and k-2 they read from (hex3d.cu wait_prev)
+        const bool chain = f3_chain && !p.pre_launch && !p.mir[0] && !p.mir[1];
+        if (chain) {
+          const int64_t k = &l - p.launches.data();
+          for (int q = 0; q < 2; ++q) {
+            if (k - 1 - q < 0) continue;
+            const Launch& pl = p.launches[(size_t)(k - 1 - q)];
+            Fast3DPrev& pv = a.prev[q];
+            pv.flags = reinterpret_cast<const int*>(ws + p.flag_off) + pl.flag_first;
+            pv.done = reinterpret_cast<const unsigned long long*>(ws + p.counter_off) + p.n_counters + pl.counter_idx;
+            pv.tau0 = pl.tau0;
+            pv.S0_lo = pl.S0_lo;
+            pv.S0_hi = pl.S0_hi;
+            pv.row_off = pl.row_off;
+            pv.S1_lo = pl.Slo[0];
+            pv.n1 = pl.Shi[0] - pl.Slo[0] + 1;
+            pv.S2_lo = pl.Slo[1];
+            pv.n2 = pl.Shi[1] - pl.Slo[1] + 1;
+          }
+          a.pdl = 1;
+          a.done = reinterpret_cast<unsigned long long*>(ws + p.counter_off) + p.n_counters + l.counter_idx;
+        }
         HEXS_CUDA(launch_fast3d(p.variant, a, grid, s), "stencil_run: fast3d kernel launch");
       } else {
         GenericArgs g{};

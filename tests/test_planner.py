@@ -216,7 +216,7 @@ def test_naive_and_auto_executor_selection():
     p = Plan(Stencil("star2d5", (64, 64)), 8)
     assert p.info["fast_kernel"] == 1  # a compiled variant, the tile model's choice for this grid
     p = Plan(Stencil("star2d5", (8192, 8192)), 8)
-    assert p.info["fast_kernel"] == 1 and p.info["h"] == 3 and p.info["w0"] == 7
+    assert p.info["fast_kernel"] == 1 and (p.info["h"], p.info["w0"]) == (2, 7)  # tile model, round 2
     p = Plan(Stencil("star2d5", (64, 64)), 8, h=2, w0=2)   # no specialised instantiation
     assert p.info["fast_kernel"] == 0
     assert p.workspace_bytes >= 64 * 64 * 4
