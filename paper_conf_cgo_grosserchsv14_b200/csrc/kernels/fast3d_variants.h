@@ -25,5 +25,6 @@
   X(12, 0, float, K_STAR3D7, 3, 5, 32, 1, 1)    \
   X(13, 0, float, K_STAR3D7, 2, 7, 16, 2, 1)    \
   X(14, 0, float, K_STAR3D7, 1, 3, 32, 2, 1)    \
-  X(15, 0, float, K_STAR3D7, 2, 7, 32, 1, 2)
-#define HEXS_FAST3D_COUNT 16
+  X(15, 0, float, K_STAR3D7, 2, 7, 32, 1, 2)    \
+  X(16, 0, float, K_STAR3D7, 3, 7, 16, 1, 1)
+#define HEXS_FAST3D_COUNT 17

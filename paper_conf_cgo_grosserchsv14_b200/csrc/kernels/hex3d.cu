@@ -101,7 +101,8 @@ template <typename T, int Q, int NY> struct Lay {
   static constexpr int EDGE_OFF = al128((CARRY_OFF + Q * CARRY) * (int)sizeof(T)) / (int)sizeof(T);
   static constexpr int BUF = al128((EDGE_OFF + Q * CARRY) * (int)sizeof(T)) / (int)sizeof(T);
   static constexpr size_t SMEM = 2 * (size_t)BUF * sizeof(T);
-  static_assert(SMEM + 1024 <= 227 * 1024, "two level buffers must fit the 227 KB opt-in shared memory");
+  static constexpr bool FITS = SMEM + 1024 <= 227 * 1024;  // two level buffers in the 227 KB opt-in
+  static_assert(FITS || HEXS_F3_NX != 32, "two level buffers must fit the 227 KB opt-in shared memory");
   static constexpr uint32_t FIRST_BYTES = (uint32_t)(Q * (MAIN + LINES + 2 * CARRY) * sizeof(T));
   static constexpr uint32_t CARRY_BYTES = (uint32_t)(Q * (LINES + 2 * CARRY) * sizeof(T));
   static constexpr uint32_t ROW_BYTES = (uint32_t)(MAIN * sizeof(T));
@@ -839,6 +840,9 @@ static bool encode(CUtensorMap* map, void* base, const Fast3DArgs& a, uint32_t b
 template <typename T, int KIND, int H, int W0, int NY, int MINB, int ZS, bool MIR>
 cudaError_t launch_t(const Fast3DArgs& a, cudaStream_t s) {
   using LY = Lay<T, Hex<H, W0>::Q, NY>;
+  if constexpr (!LY::FITS) {
+    return cudaErrorInvalidValue;  // (NX = 64 experiment builds: this tile's buffers do not fit)
+  } else {
   constexpr int NT = ZS * NY * NQ + 32;  // compute threads + the producer warp
   static DeviceMemo<int> memo;  // per device: smem opt-in + persistent grid size
   constexpr size_t smem = LY::SMEM;
@@ -866,8 +870,9 @@ cudaError_t launch_t(const Fast3DArgs& a, cudaStream_t s) {
   }
   const int64_t items = (a.S0_hi - a.S0_lo + 1) * a.n1 * a.n2;
   const int gsz = (int)(items < grid ? items : grid);
-  if (a.pdl) {
-    // chained launch: may start while the previous launch drains (its tiles wait on flags)
+  if (a.pdl && a.prev[0].flags) {
+    // chained launch: may start while the previous launch drains (its tiles wait on flags); the
+    // run's first launch follows the flag reset (a memset) strictly
     cudaLaunchConfig_t cfg = {};
     cfg.gridDim = dim3((unsigned)gsz);
     cfg.blockDim = dim3((unsigned)NT);
@@ -882,6 +887,7 @@ cudaError_t launch_t(const Fast3DArgs& a, cudaStream_t s) {
   }
   kern<<<gsz, NT, smem, s>>>(a, m);
   return cudaGetLastError();
+  }
 }
 
 }  // namespace fast3d
