@@ -29,6 +29,7 @@
 #include "../stencil_ops.cuh"
 #include "devcache.h"
 #include "launch.h"
+#include "tma.cuh"
 
 namespace hexs {
 namespace fdtd {
@@ -58,8 +59,8 @@ constexpr int NT = RP * C;
 template <typename T>
 size_t smem_bytes(int W) {
   // three fields' ring rows, plus (unrolled kernel) RP + 2 padding rows that the row slots past a
-  // level's last row may read, plus one trash word per lane that their stores go to
-  return ((size_t)3 * (W + 2) * RC + (size_t)(RP + 2) * RC + 32) * sizeof(T);
+  // level's last row may read (their stores are predicated off)
+  return ((size_t)3 * (W + 2) * RC + (size_t)(RP + 2) * RC) * sizeof(T);
 }
 
 __device__ __forceinline__ void cp_async16(void* dst, const void* src, bool valid) {
@@ -93,6 +94,15 @@ template <int H, int W0> struct FHex {
     return h1 < h2 ? h1 : h2;
   }
 };
+// predicated shared store (no select, no branch): the unrolled kernel's masked row slots
+__device__ __forceinline__ void sts_if(bool p, float* a, float v) {
+  asm volatile("{\n.reg .pred q;\nsetp.ne.b32 q, %0, 0;\n@q st.shared.f32 [%1], %2;\n}\n" ::"r"((int)p), "r"(smem_u32(a)),
+               "f"(v));
+}
+__device__ __forceinline__ void sts_if(bool p, double* a, double v) {
+  asm volatile("{\n.reg .pred q;\nsetp.ne.b32 q, %0, 0;\n@q st.shared.f64 [%1], %2;\n}\n" ::"r"((int)p), "r"(smem_u32(a)),
+               "d"(v));
+}
 template <int A, int N, class F>
 __device__ __forceinline__ void static_for(F&& f) {
   if constexpr (A < N) {
@@ -176,6 +186,7 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
   const int k_last = (int)((N1 - 1 + g.a_hi) / C);
   for (int blk = 0; blk < NB - 1; ++blk) stage(blk);
   const int col = tid & (C - 1), rpar = tid / C;  // column, row part
+  const int zrr = (int)(-i0) - rpar, nrr = (int)(N0 - 1 - i0) - rpar;  // (unrolled kernel) edge rows
   T* const rex = ring + (size_t)(0 * R + 1) * RC;  // row b of a field at r.. + b * RC + ring column
   T* const rey = ring + (size_t)(1 * R + 1) * RC;
   T* const rhz = ring + (size_t)(2 * R + 1) * RC;
@@ -196,7 +207,7 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
         // hz[j-1] for j >= 1, hz[i][j] ex[j+1] / ey[i+1] inside the grid; staging zero-fills
         // them) -- so only the in-grid cells a statement never updates (ey row 0, ex column 0,
         // hz row N0-1 and column N1-1, the oracle's loop bounds) and the row slots past the
-        // level's last row are masked: one compare per slot, no table reads, no branches.
+        // level's last row are masked: one compare per slot and a predicated store.
         const int j = k * C - a + col;
         const int cj = (int)((unsigned)(j + C) % (unsigned)RC);
         bool lvok = true;  // column / last-slot conditions of this level
@@ -204,44 +215,42 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
         if constexpr (st == 2) lvok = j != (int)N1 - 1;
         constexpr int RR = HX::W + 2;  // ring rows per field (compile-time: immediate offsets)
         T* const fb = ring + (LO + 1 + rpar) * RC + cj;  // field 0 (ex), row LO + rpar
-        T* const trash = ring + (3 * RR + RP + 2) * RC + (tid & 31);
         constexpr int LASTLIM = HI - LO - RP * (M - 1);  // the last slot exists for rpar <= LASTLIM
         const bool lastok = rpar <= LASTLIM;
-        auto slot_ok = [&](int m, int b) {
+        // row b = LO + RP m + rpar is global row 0 (ey) / N0-1 (hz) iff LO + RP m == zrr / nrr:
+        // one compare with an immediate per slot
+        auto slot_ok = [&](int m) {
           bool ok = lvok && (m < M - 1 || lastok);
-          if (st == 0) ok = ok && (b + (int)i0 != 0);
-          if (st == 2) ok = ok && (b + (int)i0 != (int)N0 - 1);
+          if (st == 0) ok = ok && (LO + RP * m != zrr);
+          if (st == 2) ok = ok && (LO + RP * m != nrr);
           return ok;
         };
         if constexpr (st == 0) {  // ey[i][j] -= ce * (hz[i][j] - hz[i-1][j])
 #pragma unroll
           for (int m = 0; m < M; ++m) {
-            const int b = LO + rpar + RP * m;
             T* pe = fb + (RR + RP * m) * RC;
             const T* ph = fb + (2 * RR + RP * m) * RC;
             const T v = fdtd_ey<T>(*pe, ph[0], ph[-RC], cf);
-            *(slot_ok(m, b) ? pe : trash) = v;
+            sts_if(slot_ok(m), pe, v);
           }
         } else if constexpr (st == 1) {  // ex[i][j] -= ce * (hz[i][j] - hz[i][j-1])
           const int dm = cj == 0 ? RC - 1 : -1;  // column j-1 in the ring
 #pragma unroll
           for (int m = 0; m < M; ++m) {
-            const int b = LO + rpar + RP * m;
             T* px = fb + (RP * m) * RC;
             const T* ph = fb + (2 * RR + RP * m) * RC;
             const T v = fdtd_ex<T>(*px, ph[0], ph[dm], cf);
-            *(slot_ok(m, b) ? px : trash) = v;
+            sts_if(slot_ok(m), px, v);
           }
         } else {  // hz[i][j] -= ch * (((ex[i][j+1] - ex[i][j]) + ey[i+1][j]) - ey[i][j])
           const int dp = cj == RC - 1 ? 1 - RC : 1;  // column j+1 in the ring
 #pragma unroll
           for (int m = 0; m < M; ++m) {
-            const int b = LO + rpar + RP * m;
             T* ph = fb + (2 * RR + RP * m) * RC;
             const T* px = fb + (RP * m) * RC;
             const T* pe = fb + (RR + RP * m) * RC;
             const T v = fdtd_hz<T>(*ph, px[dp], px[0], pe[RC], pe[0], cf);
-            *(slot_ok(m, b) ? ph : trash) = v;
+            sts_if(slot_ok(m), ph, v);
           }
         }
         // ey (tau = 3t) and ex (3t + 1) read only hz of step t-1 and write different fields:

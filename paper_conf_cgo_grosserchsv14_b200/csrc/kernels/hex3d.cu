@@ -58,7 +58,13 @@
 namespace hexs {
 namespace fast3d {
 
-constexpr int NX = kFast3DNX;  // tile columns (x)
+// tile columns (x) of the instantiation this object carries (fast3d_variants.h)
+template <int ID> struct VariantNX;
+#define HEXS_F3_NXOF(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_, NX_) \
+  template <> struct VariantNX<id> { static constexpr int value = NX_; };
+HEXS_FAST3D_VARIANTS(HEXS_F3_NXOF)
+#undef HEXS_F3_NXOF
+constexpr int NX = VariantNX<HEXS_F3_VARIANT>::value;
 constexpr int NXP = NX + 4;    // shared-memory line pitch (spreads the per-line edge loads over banks)
 constexpr int NQ = NX / 4;     // column quads: one 8-lane group
 constexpr int SIGMA = 4;       // x skew per level
@@ -101,8 +107,7 @@ template <typename T, int Q, int NY> struct Lay {
   static constexpr int EDGE_OFF = al128((CARRY_OFF + Q * CARRY) * (int)sizeof(T)) / (int)sizeof(T);
   static constexpr int BUF = al128((EDGE_OFF + Q * CARRY) * (int)sizeof(T)) / (int)sizeof(T);
   static constexpr size_t SMEM = 2 * (size_t)BUF * sizeof(T);
-  static constexpr bool FITS = SMEM + 1024 <= 227 * 1024;  // two level buffers in the 227 KB opt-in
-  static_assert(FITS || HEXS_F3_NX != 32, "two level buffers must fit the 227 KB opt-in shared memory");
+  static_assert(SMEM + 1024 <= 227 * 1024, "two level buffers must fit the 227 KB opt-in shared memory");
   static constexpr uint32_t FIRST_BYTES = (uint32_t)(Q * (MAIN + LINES + 2 * CARRY) * sizeof(T));
   static constexpr uint32_t CARRY_BYTES = (uint32_t)(Q * (LINES + 2 * CARRY) * sizeof(T));
   static constexpr uint32_t ROW_BYTES = (uint32_t)(MAIN * sizeof(T));
@@ -840,9 +845,6 @@ static bool encode(CUtensorMap* map, void* base, const Fast3DArgs& a, uint32_t b
 template <typename T, int KIND, int H, int W0, int NY, int MINB, int ZS, bool MIR>
 cudaError_t launch_t(const Fast3DArgs& a, cudaStream_t s) {
   using LY = Lay<T, Hex<H, W0>::Q, NY>;
-  if constexpr (!LY::FITS) {
-    return cudaErrorInvalidValue;  // (NX = 64 experiment builds: this tile's buffers do not fit)
-  } else {
   constexpr int NT = ZS * NY * NQ + 32;  // compute threads + the producer warp
   static DeviceMemo<int> memo;  // per device: smem opt-in + persistent grid size
   constexpr size_t smem = LY::SMEM;
@@ -887,14 +889,13 @@ cudaError_t launch_t(const Fast3DArgs& a, cudaStream_t s) {
   }
   kern<<<gsz, NT, smem, s>>>(a, m);
   return cudaGetLastError();
-  }
 }
 
 }  // namespace fast3d
 
 // the instantiation this object carries (fast3d_variants.h, -DHEXS_F3_VARIANT=<id>)
 template <int ID> struct Sel3;
-#define HEXS_F3_SEL(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_)                         \
+#define HEXS_F3_SEL(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_, NX_)                         \
   template <> struct Sel3<id> {                                                          \
     using T = T_;                                                                        \
     static constexpr int KIND = KIND_, H = H_, W0 = W0_, NY = NY_, MINB = MINB_, ZS = ZS_; \

@@ -120,10 +120,6 @@ struct Fast3DArgs {
   int pdl;  // 1: launched with programmatic stream serialization (and lets the next launch start early)
 };
 cudaError_t launch_fast3d(int variant, const Fast3DArgs& a, int grid, cudaStream_t s);
-#ifndef HEXS_F3_NX
-#define HEXS_F3_NX 32  // (experiment builds: 64 with 16-line variants)
-#endif
-constexpr int kFast3DNX = HEXS_F3_NX;    // classical tile width along x of the 3D fast kernel
 
 // Streaming 3D kernel (kernels/stream3d.cu): hexagons over (t, y), z streamed plane by plane
 // (classical width 1, skew 1), x in strips of kStream3DNX (skew 4).  One CTA per (hexagon,

@@ -67,13 +67,13 @@ int fdtd_variant(int dtype, int h, int w0) {
   return dtype == 1 ? 1 : 0;
 }
 // 3D fast kernel: the compiled (class, dtype, h, w0) instantiations of fast3d_variants.h.
-#define HEXS_F3_DECL(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_) \
+#define HEXS_F3_DECL(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_, NX_) \
   cudaError_t launch_fast3d_v##id(const Fast3DArgs& a, cudaStream_t s);
 HEXS_FAST3D_VARIANTS(HEXS_F3_DECL)
 #undef HEXS_F3_DECL
 
 int fast3d_variant(int kind, int dtype, int h, int w0, int wy) {
-#define HEXS_F3_MATCH(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_) \
+#define HEXS_F3_MATCH(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_, NX_) \
   if (kind == KIND_ && dtype == dc && h == H_ && w0 == W0_ && (wy <= 0 || wy == NY_)) return id;
   HEXS_FAST3D_VARIANTS(HEXS_F3_MATCH)
 #undef HEXS_F3_MATCH
@@ -81,7 +81,7 @@ int fast3d_variant(int kind, int dtype, int h, int w0, int wy) {
 }
 int fast3d_variant_count() { return HEXS_FAST3D_COUNT; }
 bool fast3d_variant_info(int variant, int* kind, int* dtype, int* h, int* w0) {
-#define HEXS_F3_INFO(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_) \
+#define HEXS_F3_INFO(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_, NX_) \
   if (variant == id) {                                           \
     *kind = KIND_; *dtype = dc; *h = H_; *w0 = W0_;              \
     return true;                                                 \
@@ -91,7 +91,7 @@ bool fast3d_variant_info(int variant, int* kind, int* dtype, int* h, int* w0) {
   return false;
 }
 bool fast3d_variant_matches(int variant, int kind, int dtype, int h, int w0) {
-#define HEXS_F3_IS(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_) \
+#define HEXS_F3_IS(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_, NX_) \
   if (variant == id) return kind == KIND_ && dtype == dc && h == H_ && w0 == W0_;
   HEXS_FAST3D_VARIANTS(HEXS_F3_IS)
 #undef HEXS_F3_IS
@@ -99,16 +99,19 @@ bool fast3d_variant_matches(int variant, int kind, int dtype, int h, int w0) {
 }
 int fast3d_tile(int variant, int* wy, int* wx) {
   *wy = 0;
-#define HEXS_F3_NY(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_) \
-  if (variant == id) *wy = NY_;
+  *wx = 0;
+#define HEXS_F3_NY(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_, NX_) \
+  if (variant == id) {                                           \
+    *wy = NY_;                                                   \
+    *wx = NX_;                                                   \
+  }
   HEXS_FAST3D_VARIANTS(HEXS_F3_NY)
 #undef HEXS_F3_NY
-  *wx = kFast3DNX;
   return *wy > 0 ? 0 : -1;
 }
 cudaError_t launch_fast3d(int variant, const Fast3DArgs& a, int /*grid: persistent*/, cudaStream_t s) {
   switch (variant) {
-#define HEXS_F3_L(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_) \
+#define HEXS_F3_L(id, dc, T_, KIND_, H_, W0_, NY_, MINB_, ZS_, NX_) \
   case id: return launch_fast3d_v##id(a, s);
     HEXS_FAST3D_VARIANTS(HEXS_F3_L)
 #undef HEXS_F3_L
