@@ -154,6 +154,25 @@ def test_fast3d_tiles(h, w0):
     assert_bitexact(got, oracle.run("star3d7", g, 11), f"fast3d h={h} w0={w0}")
 
 
+# (requested w[0] -- 0: the variant table's default --, expected (y, x) tile)
+@pytest.mark.parametrize("kind,h,w0,wy,tile_yx", [("star3d7", 3, 7, 0, (16, 64)), ("star3d7", 3, 7, 32, (32, 32)),
+                                                ("star3d7", 3, 7, 8, (8, 128)), ("star3d7", 2, 7, 16, (16, 32)),
+                                                ("box3d27", 2, 7, 16, (16, 64)), ("gradient3d", 2, 7, 16, (16, 64)),
+                                                ("box3d27", 2, 7, 0, (32, 32))])
+@pytest.mark.parametrize("shape,T", [((70, 150, 140), 13), ((40, 90, 300), 9), ((19, 33, 68), 20)])
+def test_fast3d_tile_shapes(kind, h, w0, wy, tile_yx, shape, T):
+    """The 3D tile-wavefront variants of every (y, x) tile shape -- the default 16 x 64 of star3d7
+    (3, 7), 32 x 32, 8 x 128 (one line per warp), 16 x 32, and the 27-point / gradient 16 x 64 --
+    on grids spanning several tiles with ragged edges, hexagons cut at t = 0 / t = T."""
+    g = stencil_inputs.uniform(shape, seed=33)
+    tile = {"h": h, "w0": w0, "hex_dim": 0}
+    if wy:
+        tile["w"] = [wy, 0, 0]
+    got, plan = _gpu_run(kind, g, T, np.float32, **tile)
+    assert plan.executor_name == "fast3d" and tuple(plan.info["w"][:2]) == tile_yx
+    assert_bitexact(got, oracle.run(kind, g, T), f"fast3d {kind} ({h},{w0}) {tile_yx} {shape} T={T}")
+
+
 @pytest.mark.parametrize("kind,h,w0", [("star3d7", 2, 7), ("star3d7", 1, 3), ("star3d7", 3, 5), ("star3d7", 1, 7),
                                        ("star3d7", 2, 5), ("star3d7", 3, 7), ("gradient3d", 2, 7),
                                        ("gradient3d", 1, 7)])
