@@ -34,7 +34,10 @@
 namespace hexs {
 namespace fdtd {
 
-constexpr int C = 64;        // columns per chunk (= ring block)
+#ifndef HEXS_FDTD_C
+#define HEXS_FDTD_C 64
+#endif
+constexpr int C = HEXS_FDTD_C;  // columns per chunk (= ring block)
 #ifndef HEXS_FDTD_PAIR
 #define HEXS_FDTD_PAIR 1  // ey and ex of a time step in one barrier interval (unrolled kernel)
 #endif
@@ -53,7 +56,10 @@ __device__ __forceinline__ int ring_col(int j) { return (j + C) % RC; }  // j >=
 #define HEXS_FDTD_RP 4  // 2 (3 CTAs/SM) measured 228 -> 197 GUp/s
 #endif
 constexpr int RP = HEXS_FDTD_RP;  // threads per column (row parts, rows interleaved)
-constexpr int MINB = (RP == 2 || NB == 3) ? 3 : 2;  // resident CTAs per SM (shared memory: 3 fields x ring)
+#ifndef HEXS_FDTD_MINB
+#define HEXS_FDTD_MINB ((RP == 2 || NB == 3) ? 3 : 2)
+#endif
+constexpr int MINB = HEXS_FDTD_MINB;  // resident CTAs per SM (shared memory: 3 fields x ring)
 constexpr int NT = RP * C;
 
 template <typename T>

@@ -44,7 +44,8 @@
                       // the FMA pipe 2 cycles, and the pair moves are IMADs on the same pipe)
 #endif
 #ifndef HEXS_MERGE_COLP
-#define HEXS_MERGE_COLP 0  // 1 measured slower: 1514 -> 1250 GUp/s star2d5
+#define HEXS_MERGE_COLP 0  // 1 (all classes) measured slower: 1514 -> 1250 GUp/s star2d5 in round 1 (per-element
+                           // selects), 1689 -> 1624 with the round-2 repair; gradient2d merges always
 #endif
 
 namespace hexs {
@@ -93,6 +94,9 @@ struct Kernel {
   // chunk_packed; the gradient's sqrt / div have no packed form) -- off by default, measured
   // slower (HEXS_F2_2D above)
   static constexpr bool kPacked = HEXS_F2_2D && std::is_same<T, float>::value && KIND != K_GRADIENT2D;
+  // one body for column-partial chunks as well: measured faster for the gradient's small (1,1)
+  // body (472 -> 518 GUp/s), slower for star / box (1689 -> 1624, 1381 -> 1331: two bodies fit)
+  static constexpr bool kMergeColp = HEXS_MERGE_COLP || KIND == K_GRADIENT2D;
 
   struct Smem {
     uint64_t mbar[L];                 // one transaction barrier per level's In rows
@@ -530,14 +534,14 @@ struct Kernel {
       // row predicate): co-resident CTAs then share the instruction stream instead of
       // thrashing the instruction cache with two ~70 KB bodies.
       (void)rowpart;
-#if HEXS_MERGE_COLP
-      // column-partial chunks share the body too (per-element column predicate)
-      (void)colpart;
-      chunk<true, true, true, false>(g, sm, k, K, i0, cf);
-#else
-      if (colpart) chunk<true, true, true, false>(g, sm, k, K, i0, cf);
-      else chunk<true, true, false, false>(g, sm, k, K, i0, cf);
-#endif
+      if constexpr (kMergeColp) {
+        // column-partial chunks share the body too (column repair per level, store predicates)
+        (void)colpart;
+        chunk<true, true, true, false>(g, sm, k, K, i0, cf);
+      } else {
+        if (colpart) chunk<true, true, true, false>(g, sm, k, K, i0, cf);
+        else chunk<true, true, false, false>(g, sm, k, K, i0, cf);
+      }
 #else
       if (rowpart) {
         if (colpart) chunk<true, true, true, false>(g, sm, k, K, i0, cf);
