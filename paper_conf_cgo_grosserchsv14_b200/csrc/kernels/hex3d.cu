@@ -48,6 +48,10 @@
 #ifndef HEXS_F3_UNROLL
 #define HEXS_F3_UNROLL 1  // 0: rolled star sweeps (smaller code; measured equal or slower)
 #endif
+#ifndef HEXS_F3_EARLY_IN
+#define HEXS_F3_EARLY_IN 0  // 1: In rows of a tile's levels issued at its start (even) / with level 1 (odd):
+                            // measured neutral (heat-3D 592 vs 597, 27-point 367 vs 370), parity green
+#endif
 #ifndef HEXS_F3_LEAD
 #define HEXS_F3_LEAD 1  // window rows loaded ahead of the shuffled row (2, 3 measured 544, 545 vs 551)
 #endif
@@ -303,6 +307,7 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
   constexpr int NC = ZS * NY * NQ, NCW = NC / 32;  // compute threads / warps; warp NCW produces
   __shared__ __align__(8) uint64_t full[2];   // buffer filled (producer arrival + TMA bytes)
   __shared__ __align__(8) uint64_t empty[2];  // buffer consumed (one arrival per compute warp)
+  __shared__ __align__(8) uint64_t inbar[2 * H + 2];  // early In rows of level a (full-time launches)
   __shared__ long long item_s[2][3];          // tile ring (S0, q1, q2); S0 < 0: no more work
   const int tid = threadIdx.x;
   const int zpart = tid / (NY * NQ);                             // row part (< ZS; producer: ZS)
@@ -310,6 +315,8 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
   const int64_t n1 = g.n1, n2 = g.n2, ns0 = g.S0_hi - g.S0_lo + 1, n_items = ns0 * n1 * n2;
   const int64_t N0 = g.N0, N1 = g.N1, N2 = g.N2, plane = N1 * N2;
   const int a_lo = g.a_lo, a_hi = g.a_hi;
+  // In rows issued early (full-time launches; HEXS_F3_EARLY_IN=0 at build time: with the carries)
+  const bool early_in = HEXS_F3_EARLY_IN && a_lo == 0 && a_hi == 2 * H + 1;
 
   // per-thread window lines k = 0..2 (input-frame line ly + k): element offset in a buffer
   // at buffer row 0, and the row pitch of the area they live in
@@ -339,6 +346,7 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
     mbar_init(&full[1], 1);
     mbar_init(&empty[0], NCW);
     mbar_init(&empty[1], NCW);
+    for (int a = 0; a < 2 * H + 2; ++a) mbar_init(&inbar[a], 1);
     mbar_fence_init();
   }
   __syncthreads();
@@ -396,7 +404,7 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
     lo2[0] = need_lo; n2_[0] = need_lo < clo ? clo - need_lo : 0;
     lo2[1] = chi + 1; n2_[1] = need_hi > chi ? need_hi - chi : 0;
   };
-  auto issue_in = [&](const long long* it, int a) {
+  auto issue_in = [&](const long long* it, int a, uint64_t* bar) {
     int64_t i0;
     int X0, Y0;
     tile_origin(it, i0, X0, Y0);
@@ -409,10 +417,10 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
         const int bb = lo2[s] + k;
         T* dst = buf_of(b) + (bb + 1) * LY::MAIN;
         if (nn[s] - k >= 2) {
-          tma_3d(dst, &mp.in2[par], xo + 4, yo + 1, (int)(i0 + bb), &full[b]);
+          tma_3d(dst, &mp.in2[par], xo + 4, yo + 1, (int)(i0 + bb), bar);
           k += 2;
         } else {
-          tma_3d(dst, &mp.in1[par], xo + 4, yo + 1, (int)(i0 + bb), &full[b]);
+          tma_3d(dst, &mp.in1[par], xo + 4, yo + 1, (int)(i0 + bb), bar);
           k += 1;
         }
       }
@@ -525,6 +533,15 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
               F3_TR(4, ptile, a);
             }
             issue_first(it, a);
+            // early In rows (full-time launches): every even level's In rows land in buffer
+            // b(0) rows no level before it reads or writes (the hexagon widens by one row per
+            // side per level), so they go out with the first fill, on their own barriers
+            if (early_in) {
+              for (int a2 = 2; a2 <= H + 1; a2 += 2) {
+                mbar_arrive_expect_tx(&inbar[a2], in_bytes(a2));
+                issue_in(it, a2, &inbar[a2]);
+              }
+            }
           } else {
             if (a == a_lo + 1) {  // predecessors complete: their carries are in global memory
               F3_TR(3, ptile, a);
@@ -543,8 +560,20 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
               F3_TR(4, ptile, a);
               F3_TM(2);
             }
-            mbar_arrive_expect_tx(&full[b], LY::CARRY_BYTES + (a <= H + 1 ? in_bytes(a) : 0u));
-            if (a <= H + 1) issue_in(it, a);
+            if (early_in) {
+              // the odd levels' In rows go out once the previous tile's last level released
+              // buffer b(1), i.e. with level 1's carries
+              if (a == 1) {
+                for (int a2 = 1; a2 <= H + 1; a2 += 2) {
+                  mbar_arrive_expect_tx(&inbar[a2], in_bytes(a2));
+                  issue_in(it, a2, &inbar[a2]);
+                }
+              }
+              mbar_arrive_expect_tx(&full[b], LY::CARRY_BYTES);
+            } else {
+              mbar_arrive_expect_tx(&full[b], LY::CARRY_BYTES + (a <= H + 1 ? in_bytes(a) : 0u));
+              if (a <= H + 1) issue_in(it, a, &full[b]);
+            }
             issue_carries(it, a);
           }
           ++fills[b];
@@ -600,6 +629,7 @@ __global__ void __launch_bounds__(ZS * NY * NQ + 32, MINB) fast3d_kernel(const _
           const int dR = R0 - LO;
           if (tid == 0) F3_TR(5, ctile, A);
           if (A != a_lo) mbar_wait_parity(&full[b], (ph >> b) & 1u);
+          if (early_in && A >= 1 && A <= H + 1) mbar_wait_parity(&inbar[A], (uint32_t)(ctile & 1));
           ph ^= 1u << b;
           F3_TM(0);
           named_barrier_sync(1, NC);  // level A-1's buffer writes visible to every compute warp
