@@ -5,7 +5,8 @@
 // compiled from hex3d.cu with -DHEXS_F3_VARIANT=id into its own object (parallel build).
 // The first entry of a (class, dtype, h, w0) is its default: star3d7 fp32 (3, 7) runs 16 x 64 (y, x)
 // tiles (596 vs 567 GUp/s for 32 x 32 on heat-3D 512^3; 8 x 128: 427; the 27-point and gradient sweeps
-// measured equal or slower at 16 x 64).  (2, 7) is the default 3D tile (Table 4's h = 2); the star3d7 fp32
+// measured equal or slower at 16 x 64; deeper / wider hexagons at 16 x 64, compiled for the sweep and
+// removed: (4,7) 441, (3,9) 571 GUp/s, both bit-exact).  (2, 7) is the default 3D tile (Table 4's h = 2); the star3d7 fp32
 // shapes serve the tile sweep and the tests; the long gradient / 27-point expressions split each
 // column's rows over 2 threads (ZS = 2: 16 compute warps hide their latency; gradient 232 -> 321
 // GUp/s); a
