@@ -38,6 +38,9 @@ namespace fdtd {
 #define HEXS_FDTD_C 64
 #endif
 constexpr int C = HEXS_FDTD_C;  // columns per chunk (= ring block)
+#ifndef HEXS_FDTD_BLOCKROWS
+#define HEXS_FDTD_BLOCKROWS 1  // ey / hz levels: contiguous row blocks per thread (register reuse)
+#endif
 #ifndef HEXS_FDTD_PAIR
 #define HEXS_FDTD_PAIR 1  // ey and ex of a time step in one barrier interval (unrolled kernel)
 #endif
@@ -231,7 +234,35 @@ __global__ void __launch_bounds__(NT, MINB) fdtd_kernel(const __grid_constant__ 
           if (st == 2) ok = ok && (LO + RP * m != nrr);
           return ok;
         };
-        if constexpr (st == 0) {  // ey[i][j] -= ce * (hz[i][j] - hz[i-1][j])
+        // Block rows (HEXS_FDTD_BLOCKROWS): thread rpar takes rows LO + rpar M + m, so the
+        // row neighbours a statement reads (hz[i-1] for ey, ey[i+1] for hz) are the previous /
+        // next slot's own loads -- one shared load per slot fewer for ey and hz
+        const int nrow = HI - LO + 1 - rpar * M;  // valid slots m < nrow
+        T* const fbb = ring + (LO + 1 + rpar * M) * RC + cj;
+        const int zb = zrr + rpar - rpar * M, nb = nrr + rpar - rpar * M;  // edge rows as LO + m
+        if constexpr (HEXS_FDTD_BLOCKROWS && st == 0) {
+          T hprev = fbb[(2 * RR - 1) * RC];  // hz[b-1] of slot 0
+#pragma unroll
+          for (int m = 0; m < M; ++m) {
+            T* pe = fbb + (RR + m) * RC;
+            const T hb = fbb[(2 * RR + m) * RC];
+            const T v = fdtd_ey<T>(*pe, hb, hprev, cf);
+            hprev = hb;
+            sts_if(lvok && m < nrow && LO + m != zb, pe, v);
+          }
+        } else if constexpr (HEXS_FDTD_BLOCKROWS && st == 2) {
+          const int dp = cj == RC - 1 ? 1 - RC : 1;  // column j+1 in the ring
+          T enext = fbb[RR * RC];  // ey[b] of slot 0
+#pragma unroll
+          for (int m = 0; m < M; ++m) {
+            T* ph = fbb + (2 * RR + m) * RC;
+            const T* px = fbb + m * RC;
+            const T eb = enext;
+            enext = fbb[(RR + m + 1) * RC];  // ey[b+1] = the next slot's ey[b]
+            const T v = fdtd_hz<T>(*ph, px[dp], px[0], enext, eb, cf);
+            sts_if(lvok && m < nrow && LO + m != nb, ph, v);
+          }
+        } else if constexpr (st == 0) {  // ey[i][j] -= ce * (hz[i][j] - hz[i-1][j])
 #pragma unroll
           for (int m = 0; m < M; ++m) {
             T* pe = fb + (RR + RP * m) * RC;
