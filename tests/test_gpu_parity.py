@@ -111,7 +111,10 @@ def test_fdtd(dtype, executor):
 @pytest.mark.parametrize("dtype", [np.float32, np.float64])
 @pytest.mark.parametrize("shape,T,h,w0", [((64, 80), 9, 0, 0), ((101, 260), 17, 0, 0), ((37, 132), 13, 2, 0),
                                           ((90, 72), 11, 5, 3), ((70, 200), 25, 3, 1), ((130, 68), 8, 8, 4),
-                                          ((9, 4), 5, 0, 0), ((300, 324), 30, 5, 5)])
+                                          ((9, 4), 5, 0, 0), ((300, 324), 30, 5, 5),
+                                          # the compile-time unrolled (11, 5) kernel: several
+                                          # hexagons, both row edges, ragged chunks, full and cut launches
+                                          ((200, 330), 40, 11, 5), ((57, 1000), 19, 11, 5)])
 def test_fdtd_fast_kernel(dtype, shape, T, h, w0):
     """The shared-memory-ring FDTD kernel (kernels/fdtd.cu): ragged chunk tails, hexagons cut
     by the grid, partial first/last launches, tiny grids -- bit-exact against the oracle."""
