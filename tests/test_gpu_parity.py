@@ -114,7 +114,7 @@ def test_fdtd(dtype, executor):
                                           ((9, 4), 5, 0, 0), ((300, 324), 30, 5, 5),
                                           # the compile-time unrolled (11, 5) kernel: several
                                           # hexagons, both row edges, ragged chunks, full and cut launches
-                                          ((200, 330), 40, 11, 5), ((57, 1000), 19, 11, 5)])
+                                          ((200, 332), 40, 11, 5), ((57, 1000), 19, 11, 5)])
 def test_fdtd_fast_kernel(dtype, shape, T, h, w0):
     """The shared-memory-ring FDTD kernel (kernels/fdtd.cu): ragged chunk tails, hexagons cut
     by the grid, partial first/last launches, tiny grids -- bit-exact against the oracle."""
