@@ -39,6 +39,9 @@
 #ifndef HEXS_MERGE_ROWP
 #define HEXS_MERGE_ROWP 1
 #endif
+#ifndef HEXS_2D_DRIFT
+#define HEXS_2D_DRIFT 0  // 1: no CTA barrier per level -- tail hand-off by mbarrier, last-arriver refill
+#endif
 #ifndef HEXS_F2_2D
 #define HEXS_F2_2D 0  // 1 measured slower: heat2d5 1551 -> 1379 GUp/s, box2d9 1151 -> 946 (FADD2 holds
                       // the FMA pipe 2 cycles, and the pair moves are IMADs on the same pipe)
@@ -100,6 +103,8 @@ struct Kernel {
 
   struct Smem {
     uint64_t mbar[L];                 // one transaction barrier per level's In rows
+    uint64_t tailbar[2][L][NW];       // (drift mode) tail of [chunk parity][level][warp] written
+    unsigned cnt[L];                  // (drift mode) warps done with a level's In rows
     T tail[2][L][NW][Q][2];           // [chunk parity][level][warp][row][2 last columns]
     alignas(16) T inrows[NIN][SW];    // In rows of the current chunk (TMA-staged)
   };
@@ -216,6 +221,14 @@ struct Kernel {
         static_assert(!TCUT, "TMA staging runs full-time tiles only");
         if constexpr (n_in(a) > 0) mbar_wait_parity(&sm.mbar[a], (uint32_t)(k & 1));
       }
+      // drift mode: the previous warp's (previous chunk's last warp's) level a-1 tail is written
+      if constexpr (HEXS_2D_DRIFT && TMA && a > 0) {
+        if (warp > 0) {
+          mbar_wait_parity(&sm.tailbar[k & 1][a - 1][warp - 1], (uint32_t)((k >> 1) & 1));
+        } else if (k > 0) {
+          mbar_wait_parity(&sm.tailbar[(k - 1) & 1][a - 1][NW - 1], (uint32_t)(((k - 1) >> 1) & 1));
+        }
+      }
 
       // ---- (2)-(5) rows ascending: inputs just in time, compute, copy out, tail ----
       const int pw = warp == 0 ? NW - 1 : warp - 1;
@@ -329,8 +342,28 @@ struct Kernel {
             sm.tail[k & 1][a][warp][q][0] = out[q][V - 2];
             sm.tail[k & 1][a][warp][q][1] = out[q][V - 1];
           }
+          if constexpr (HEXS_2D_DRIFT && TMA) mbar_arrive(&sm.tailbar[k & 1][a][warp]);  // release
         }
       }
+      if constexpr (HEXS_2D_DRIFT && TMA) {
+        // ---- refill without a CTA barrier: the last warp done with level a's In rows issues
+        // chunk k+1's (its fence orders every warp's reads before the async-proxy writes) ----
+        if constexpr (n_in(a) > 0) {
+          __syncwarp();
+          if (lane == 0) {
+            __threadfence_block();
+            const unsigned old = atomicAdd(&sm.cnt[a], 1u);
+            if (old == NW - 1) {
+              sm.cnt[a] = 0u;
+              __threadfence_block();
+              if (k + 1 < K) {
+                fence_proxy_async_smem();
+                issue_level(g, sm, k + 1, a, i0);
+              }
+            }
+          }
+        }
+      } else {
       __syncthreads();
       // ---- refill: the consumed slots of level a take chunk k+1's In rows ----
       if constexpr (TMA && n_in(a) > 0) {
@@ -338,6 +371,7 @@ struct Kernel {
           fence_proxy_async_smem();
           issue_level(g, sm, k + 1, a, i0);
         }
+      }
       }
       // ---- (6) the outputs become the next level's inputs ----
 #pragma unroll
@@ -520,6 +554,15 @@ struct Kernel {
     if (threadIdx.x == 0) {
 #pragma unroll
       for (int a = 0; a < L; ++a) mbar_init(&sm.mbar[a], 1);
+      if constexpr (HEXS_2D_DRIFT) {
+        for (int a = 0; a < L; ++a) {
+          sm.cnt[a] = 0u;
+          for (int w = 0; w < NW; ++w) {
+            mbar_init(&sm.tailbar[0][a][w], 1);
+            mbar_init(&sm.tailbar[1][a][w], 1);
+          }
+        }
+      }
       mbar_fence_init();
     }
     __syncthreads();
