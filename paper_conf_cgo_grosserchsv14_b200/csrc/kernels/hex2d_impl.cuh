@@ -40,7 +40,9 @@
 #define HEXS_MERGE_ROWP 1
 #endif
 #ifndef HEXS_2D_DRIFT
-#define HEXS_2D_DRIFT 0  // 1: no CTA barrier per level -- tail hand-off by mbarrier, last-arriver refill
+#define HEXS_2D_DRIFT 0  // 1: no CTA barrier per level -- tail hand-off by mbarrier, last-arriver refill:
+                         // bit-exact but measured slower (heat2d5 1672 -> 1212: warps serialise on
+                         // their predecessor's tail, 168 vs 147 registers)
 #endif
 #ifndef HEXS_F2_2D
 #define HEXS_F2_2D 0  // 1 measured slower: heat2d5 1551 -> 1379 GUp/s, box2d9 1151 -> 946 (FADD2 holds
