@@ -105,8 +105,10 @@ struct Kernel {
 
   struct Smem {
     uint64_t mbar[L];                 // one transaction barrier per level's In rows
+#if HEXS_2D_DRIFT
     uint64_t tailbar[2][L][NW];       // (drift mode) tail of [chunk parity][level][warp] written
     unsigned cnt[L];                  // (drift mode) warps done with a level's In rows
+#endif
     T tail[2][L][NW][Q][2];           // [chunk parity][level][warp][row][2 last columns]
     alignas(16) T inrows[NIN][SW];    // In rows of the current chunk (TMA-staged)
   };
@@ -223,14 +225,16 @@ struct Kernel {
         static_assert(!TCUT, "TMA staging runs full-time tiles only");
         if constexpr (n_in(a) > 0) mbar_wait_parity(&sm.mbar[a], (uint32_t)(k & 1));
       }
+#if HEXS_2D_DRIFT
       // drift mode: the previous warp's (previous chunk's last warp's) level a-1 tail is written
-      if constexpr (HEXS_2D_DRIFT && TMA && a > 0) {
+      if constexpr (TMA && a > 0) {
         if (warp > 0) {
           mbar_wait_parity(&sm.tailbar[k & 1][a - 1][warp - 1], (uint32_t)((k >> 1) & 1));
         } else if (k > 0) {
           mbar_wait_parity(&sm.tailbar[(k - 1) & 1][a - 1][NW - 1], (uint32_t)(((k - 1) >> 1) & 1));
         }
       }
+#endif
 
       // ---- (2)-(5) rows ascending: inputs just in time, compute, copy out, tail ----
       const int pw = warp == 0 ? NW - 1 : warp - 1;
@@ -344,10 +348,18 @@ struct Kernel {
             sm.tail[k & 1][a][warp][q][0] = out[q][V - 2];
             sm.tail[k & 1][a][warp][q][1] = out[q][V - 1];
           }
-          if constexpr (HEXS_2D_DRIFT && TMA) mbar_arrive(&sm.tailbar[k & 1][a][warp]);  // release
+#if HEXS_2D_DRIFT
+          if constexpr (TMA) mbar_arrive(&sm.tailbar[k & 1][a][warp]);  // release
+#endif
         }
       }
-      if constexpr (HEXS_2D_DRIFT && TMA) {
+#if HEXS_2D_DRIFT
+      constexpr bool kDrift = TMA;
+#else
+      constexpr bool kDrift = false;
+#endif
+      if constexpr (kDrift) {
+#if HEXS_2D_DRIFT
         // ---- refill without a CTA barrier: the last warp done with level a's In rows issues
         // chunk k+1's (its fence orders every warp's reads before the async-proxy writes) ----
         if constexpr (n_in(a) > 0) {
@@ -365,6 +377,7 @@ struct Kernel {
             }
           }
         }
+#endif
       } else {
       __syncthreads();
       // ---- refill: the consumed slots of level a take chunk k+1's In rows ----
@@ -556,15 +569,15 @@ struct Kernel {
     if (threadIdx.x == 0) {
 #pragma unroll
       for (int a = 0; a < L; ++a) mbar_init(&sm.mbar[a], 1);
-      if constexpr (HEXS_2D_DRIFT) {
-        for (int a = 0; a < L; ++a) {
-          sm.cnt[a] = 0u;
-          for (int w = 0; w < NW; ++w) {
-            mbar_init(&sm.tailbar[0][a][w], 1);
-            mbar_init(&sm.tailbar[1][a][w], 1);
-          }
+#if HEXS_2D_DRIFT
+      for (int a = 0; a < L; ++a) {
+        sm.cnt[a] = 0u;
+        for (int w = 0; w < NW; ++w) {
+          mbar_init(&sm.tailbar[0][a][w], 1);
+          mbar_init(&sm.tailbar[1][a][w], 1);
         }
       }
+#endif
       mbar_fence_init();
     }
     __syncthreads();
